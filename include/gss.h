@@ -1,0 +1,207 @@
+/*
+ * gss.h -- C ABI of the B200 GPU sample sort (libgss.so).
+ *
+ * Implements the k-way distribution pass of Leischner, Osipov & Sanders,
+ * "GPU Sample Sort" (IPDPS 2010; /root/reference/PAPER.md, cited P:<line>):
+ * sample and sort splitters (Phase 1), classify every key
+ * by a branch-free descent of the implicit splitter tree (Phase 2,
+ * Algorithm 2), prefix-sum the per-tile bucket
+ * histograms bucket-major (Phase 3), scatter keys and values into
+ * their buckets (Phase 4), recurse until buckets hold at most M
+ * keys (Algorithm 1), and finish those buckets with an
+ * in-SM merge sort built on an odd-even merge network.
+ *
+ * Conventions (all entry points):
+ *   - Keys are unsigned integers ordered by "<" (the comparator-only
+ *     contract of P:52-54: the kernels only ever evaluate less(a, b)).
+ *     Values are opaque payloads that move with their keys.
+ *   - Pointers are DEVICE pointers unless the name or comment says host.
+ *     The caller owns every buffer; the library never allocates device
+ *     memory.  `temp` is caller-provided scratch: call once with
+ *     temp == NULL to get *temp_bytes (no launch, no GPU access), then
+ *     again with at least that many bytes (256-byte aligned).
+ *   - `stream` is a cudaStream_t (NULL = the legacy default stream).  Every
+ *     call only enqueues work on it (stream ordered, asynchronous) unless
+ *     params->stats is set, in which case it synchronises the stream to
+ *     fill the statistics.
+ *   - keys_in may equal keys_out (in place); vals_in may equal vals_out.
+ *     Partial overlap, or temp overlapping an I/O buffer, is
+ *     GSS_ERROR_INVALID_VALUE.
+ *   - n == 0 succeeds without a launch.  n must be < 2^32 per call
+ *     (u32 offsets), else GSS_ERROR_NOT_SUPPORTED.
+ *   - Errors are reported only through the return code: nothing aborts,
+ *     throws or prints.  Asynchronous device faults surface at the
+ *     caller's next synchronisation as usual in CUDA.
+ *   - Output keys are the unique non-decreasing permutation of the input.
+ *     Values of equal keys may appear in any order (the sort is unstable,
+ *     P:262) but the output is deterministic for a fixed input,
+ *     parameter set and device.
+ */
+#ifndef GSS_H
+#define GSS_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum gss_status {
+  GSS_SUCCESS = 0,
+  GSS_ERROR_INVALID_VALUE = 1,   /* NULL with n>0, bad k/a/M/tile, overlapping buffers   */
+  GSS_ERROR_TEMP_TOO_SMALL = 2,  /* *temp_bytes smaller than the query returned         */
+  GSS_ERROR_NOT_SUPPORTED = 3,   /* n >= 2^32, or device is not sm_100                   */
+  GSS_ERROR_CUDA = 4,            /* a launch or runtime call failed                      */
+  GSS_ERROR_NCCL = 5,            /* reserved for the distributed layer                   */
+  GSS_ERROR_CAPACITY = 6         /* an output capacity is smaller than the result        */
+} gss_status;
+
+/* Kernel kinds, for gss_profiler_read(). */
+enum {
+  GSS_K_INIT = 0, GSS_K_SAMPLE, GSS_K_CLASSIFY, GSS_K_SCAN, GSS_K_SCATTER, GSS_K_PLAN,
+  GSS_K_SMALL_SORT, GSS_K_COPY, GSS_K_OVERFLOW, GSS_K_H2D, GSS_K_D2H, GSS_K_OTHER,
+  GSS_KERNEL_KINDS
+};
+
+/* Statistics of one call (host struct, filled only when requested). */
+typedef struct gss_stats {
+  uint32_t levels;              /* distribution levels that split >= 1 bucket            */
+  uint32_t launches;            /* kernels the call enqueued                             */
+  uint32_t levels_launched;     /* distribution levels enqueued (max_levels resolved)     */
+  uint32_t error_flags;         /* internal capacity checks; 0 means the result is valid */
+  uint64_t split_elems[16];     /* keys distributed at level l (sum of m over its buckets) */
+  uint64_t split_buckets[16];   /* buckets split at level l                              */
+  uint64_t small_buckets;       /* buckets finished by the in-SM sort                   */
+  uint64_t small_elems;         /* keys in those buckets                                 */
+  uint64_t max_small;           /* largest bucket given to the in-SM sort                */
+  uint64_t eq_buckets;          /* final equality buckets (all keys equal, R4)           */
+  uint64_t eq_elems;
+  uint64_t overflow_buckets;    /* buckets finished by the fallback after max_levels     */
+  uint64_t overflow_elems;
+} gss_stats;
+
+typedef struct gss_profiler gss_profiler;
+
+/* Tuning and method parameters; pass NULL for the per-type defaults. A zero
+ * field also selects its default. */
+typedef struct gss_params {
+  uint32_t k;               /* max buckets per split: power of 2 in [2,1024]      */
+  uint32_t oversample;      /* a; 0 -> 30                               */
+  uint64_t small_threshold; /* M: buckets with m <= M go to the in-SM sort;       */
+                            /* 0 -> the in-SM capacity of the type; at most that           */
+  uint32_t tile;            /* keys per tile T = t*l; multiple of 2048          */
+  uint32_t max_levels;      /* distribution levels launched before the fallback; 0 -> auto */
+  uint32_t k_policy;        /* 1 (default) adaptive k_b (R29), 2 = fixed k_b = k (paper)   */
+  uint32_t fill_div;        /* adaptive rule divisor f (R29); 0 -> 4              */
+  uint64_t seed;            /* sampling seed (R2); 0 -> 5489                               */
+  uint32_t flags;           /* GSS_FLAG_* below                                            */
+  uint32_t reserved;
+  gss_stats* stats;         /* optional host pointer: the call syncs and fills it          */
+  gss_profiler* profiler;   /* optional: CUDA-event time of every launch                   */
+} gss_params;
+
+#define GSS_FLAG_RECOMPUTE_IDS 1u  /* Phase 4 re-descends the tree instead of reading stored
+                                      bucket ids (the paper's choice)            */
+
+/* Human-readable name of a status code (static storage). */
+const char* gss_status_string(gss_status s);
+
+/* Library version and the per-type default parameters (host-only, no GPU). */
+uint32_t gss_version(void);
+gss_status gss_default_params(uint32_t key_bytes, uint32_t val_bytes, gss_params* out);
+
+/* ---------------------------------------------------------------------- */
+/* Sorting (Algorithm 1).  Device buffers of n elements.        */
+/* ---------------------------------------------------------------------- */
+gss_status gss_sort_u32(const uint32_t* keys_in, uint32_t* keys_out, size_t n,
+                        void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_sort_u64(const uint64_t* keys_in, uint64_t* keys_out, size_t n,
+                        void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_sort_pairs_u32(const uint32_t* keys_in, const uint32_t* vals_in,
+                              uint32_t* keys_out, uint32_t* vals_out, size_t n,
+                              void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_sort_pairs_u64(const uint64_t* keys_in, const uint64_t* vals_in,
+                              uint64_t* keys_out, uint64_t* vals_out, size_t n,
+                              void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+
+/* Descending order: the same kernels instantiated with less(a,b) = a > b,
+ * exercising the comparator-only contract. */
+gss_status gss_sort_u64_descending(const uint64_t* keys_in, uint64_t* keys_out, size_t n,
+                                   void* temp, size_t* temp_bytes, void* stream,
+                                   const gss_params* p);
+
+/* End-to-end variants: keys (and values) are HOST buffers (pinned for full
+ * speed); the call enqueues the host->device copy, the sort and the
+ * device->host copy on `stream`.  temp must also hold the device copies
+ * (the query includes them).  The output is valid after the stream is
+ * synchronised. */
+gss_status gss_sort_host_u32(const uint32_t* h_keys_in, uint32_t* h_keys_out, size_t n,
+                             void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_sort_host_u64(const uint64_t* h_keys_in, uint64_t* h_keys_out, size_t n,
+                             void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_sort_host_pairs_u32(const uint32_t* h_keys_in, const uint32_t* h_vals_in,
+                                   uint32_t* h_keys_out, uint32_t* h_vals_out, size_t n,
+                                   void* temp, size_t* temp_bytes, void* stream,
+                                   const gss_params* p);
+gss_status gss_sort_host_pairs_u64(const uint64_t* h_keys_in, const uint64_t* h_vals_in,
+                                   uint64_t* h_keys_out, uint64_t* h_vals_out, size_t n,
+                                   void* temp, size_t* temp_bytes, void* stream,
+                                   const gss_params* p);
+
+/* ---------------------------------------------------------------------- */
+/* One k-way distribution step over the whole input (Phases 1-4,           */
+/* P:251-263), regardless of M.  The partition is stable (R7).   */
+/*   vals_in/vals_out: NULL for keys only; values have the key's width.     */
+/*   splitters_out: device, capacity k-1 keys: the k_s - 1 sorted splitters */
+/*   bucket_offsets_out: device u64, capacity 2k: K+1 bucket boundaries      */
+/*   info_out: device u32[4] = { k_b, k_s, eq, K }                           */
+/* ---------------------------------------------------------------------- */
+gss_status gss_partition_u32(const uint32_t* keys_in, const uint32_t* vals_in,
+                             uint32_t* keys_out, uint32_t* vals_out, size_t n,
+                             uint32_t* splitters_out, uint64_t* bucket_offsets_out,
+                             uint32_t* info_out, void* temp, size_t* temp_bytes, void* stream,
+                             const gss_params* p);
+gss_status gss_partition_u64(const uint64_t* keys_in, const uint64_t* vals_in,
+                             uint64_t* keys_out, uint64_t* vals_out, size_t n,
+                             uint64_t* splitters_out, uint64_t* bucket_offsets_out,
+                             uint32_t* info_out, void* temp, size_t* temp_bytes, void* stream,
+                             const gss_params* p);
+
+/* ---------------------------------------------------------------------- */
+/* Building blocks of the distributed sample sort. */
+/* ---------------------------------------------------------------------- */
+/* Gather s keys of keys[0..n) at positions lo_global-keyed hashed indices:
+ * out[j] = keys[mulhi64(H(seed, level_tag, lo_global, j), n)] (R2). */
+gss_status gss_sample_u32(const uint32_t* keys, size_t n, uint64_t lo_global, uint32_t level_tag,
+                          uint64_t seed, uint32_t* out, size_t s, void* stream);
+gss_status gss_sample_u64(const uint64_t* keys, size_t n, uint64_t lo_global, uint32_t level_tag,
+                          uint64_t seed, uint64_t* out, size_t s, void* stream);
+
+/* Partition keys_in[0..n) (and values) into nspl+1 buckets by the given
+ * sorted device splitters (ties go left, R3; no equality buckets), writing
+ * the stable partition to keys_out/vals_out and the nspl+1 bucket sizes to
+ * counts_out (device u64). */
+gss_status gss_partition_by_u32(const uint32_t* keys_in, const uint32_t* vals_in,
+                                uint32_t* keys_out, uint32_t* vals_out, size_t n,
+                                const uint32_t* splitters, uint32_t nspl, uint64_t* counts_out,
+                                void* temp, size_t* temp_bytes, void* stream);
+gss_status gss_partition_by_u64(const uint64_t* keys_in, const uint64_t* vals_in,
+                                uint64_t* keys_out, uint64_t* vals_out, size_t n,
+                                const uint64_t* splitters, uint32_t nspl, uint64_t* counts_out,
+                                void* temp, size_t* temp_bytes, void* stream);
+
+/* ---------------------------------------------------------------------- */
+/* Profiling: CUDA events around every launch of the calls that carry the */
+/* profiler in their params.  Read after the stream has been synchronised. */
+/* ---------------------------------------------------------------------- */
+gss_status gss_profiler_create(gss_profiler** out);
+gss_status gss_profiler_destroy(gss_profiler* p);
+gss_status gss_profiler_reset(gss_profiler* p);
+/* ms[GSS_KERNEL_KINDS] and launches[GSS_KERNEL_KINDS]: host arrays */
+gss_status gss_profiler_read(gss_profiler* p, double* ms, uint64_t* launches);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* GSS_H */

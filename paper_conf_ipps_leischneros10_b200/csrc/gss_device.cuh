@@ -1,0 +1,367 @@
+// gss_device.cuh -- device-side data structures and primitives of the B200
+// GPU sample sort (Leischner, Osipov & Sanders, IPDPS 2010; PAPER.md P:<line>).
+//
+// Written for sm_100a.  Everything here is integer work: unsigned compares,
+// moves, counting and scans; no tensor cores (nothing is a contraction).
+#pragma once
+
+#include <cstdint>
+#include <type_traits>
+#include <cuda_runtime.h>
+
+namespace gss {
+
+constexpr int kNumClasses = 4;        // in-SM sort size classes (2K, 4K, 8K, 16K keys)
+constexpr int kMaxLevels = 16;        // distribution levels launched at most
+constexpr int kItems = 16;            // keys per thread in the in-SM sort
+constexpr uint32_t kFull = 0xffffffffu;
+
+enum Buf : uint32_t { BUF_IN = 0, BUF_TMP = 1, BUF_OUT = 2 };
+enum Mode : uint32_t { MODE_SORT = 0, MODE_PARTITION = 1, MODE_PARTITION_BY = 2 };
+
+struct NoVal {};
+template <class V> constexpr bool kHasVal = !std::is_same<V, NoVal>::value;
+
+// Keys are ordered only through a comparator.
+struct Less {
+  template <class T> __device__ __forceinline__ bool operator()(const T& a, const T& b) const { return a < b; }
+};
+struct Greater {
+  template <class T> __device__ __forceinline__ bool operator()(const T& a, const T& b) const { return b < a; }
+};
+
+// A bucket being split at some level (one row of the paper's k x p table
+// per tile).
+struct Bucket {
+  uint32_t lo, m;          // range [lo, lo+m) of the level's source buffer
+  uint32_t tile_start;     // first level-global tile index
+  uint32_t ntiles;         // p = ceil(m / T)
+  uint32_t kb;             // k_b: buckets asked for (R29)
+  uint32_t ks;             // range buckets: k_b, or k_b/2 in equality mode (R4)
+  uint32_t K;              // bucket ids: ks, or 2 ks - 1 in equality mode
+  uint32_t eq;             // equality mode
+  uint32_t hist_base;      // start of this bucket's K x ntiles histogram (bucket-major)
+  uint32_t spl_base;       // start of its splitter storage: tree[kb] then sorted spl[kb]
+  uint32_t clamp;          // partition_by: ids are min(b, K-1)
+  uint32_t pad;
+};
+
+struct Item {              // a final bucket (small sort / copy / overflow work)
+  uint32_t lo, m, buf, pad;
+};
+
+struct LevelCounters {
+  uint32_t num_buckets, num_tiles, hist_alloc, spl_alloc;
+  unsigned long long split_elems;
+};
+
+struct Counters {
+  LevelCounters lvl[kMaxLevels + 1];
+  uint32_t small_count[kNumClasses];
+  uint32_t copy_count, ovf_count, err, pad;
+  unsigned long long small_elems, max_small, eq_buckets, eq_elems, ovf_elems;
+};
+
+// Everything a kernel needs, passed by value.
+template <class Key, class Val, class IdT>
+struct Ctx {
+  const Key* kin; Key* ktmp; Key* kout;
+  const Val* vin; Val* vtmp; Val* vout;
+  IdT* ids;
+  Counters* cnt;
+  Bucket* bk[2];
+  uint32_t* tile_bucket[2];
+  uint32_t* hist[2];
+  Key* spl[2];
+  Item* small[kNumClasses];
+  Item* copy;
+  Item* ovf;
+  uint32_t* scan_part;
+  const Key* given_spl;              // MODE_PARTITION_BY
+  uint32_t given_nspl;
+  uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0;
+  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf;
+  uint32_t cap_small[kNumClasses];
+  uint32_t class_cap[kNumClasses];
+  uint64_t seed;
+
+  __device__ __forceinline__ uint32_t dst(uint32_t l) const {
+    uint32_t other = dst0 == BUF_TMP ? BUF_OUT : BUF_TMP;
+    return (l & 1) ? other : dst0;
+  }
+  __device__ __forceinline__ uint32_t src(uint32_t l) const { return l == 0 ? src0 : dst(l - 1); }
+  __device__ __forceinline__ const Key* keys(uint32_t b) const {
+    return b == BUF_IN ? kin : (b == BUF_TMP ? ktmp : kout);
+  }
+  __device__ __forceinline__ Key* wkeys(uint32_t b) const { return b == BUF_TMP ? ktmp : kout; }
+  __device__ __forceinline__ const Val* vals(uint32_t b) const {
+    return b == BUF_IN ? vin : (b == BUF_TMP ? vtmp : vout);
+  }
+  __device__ __forceinline__ Val* wvals(uint32_t b) const { return b == BUF_TMP ? vtmp : vout; }
+};
+
+// --------------------------------------------------------------------------
+// Sample positions: SplitMix64 counter hash (R2, replacing the paper's LCG
+// seeded by a CPU Mersenne Twister).
+// --------------------------------------------------------------------------
+__device__ __forceinline__ uint64_t splitmix64(uint64_t x) {
+  uint64_t z = x + 0x9E3779B97F4A7C15ull;
+  z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+  z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+  return z ^ (z >> 31);
+}
+__device__ __forceinline__ uint64_t sample_pos(uint64_t seed, uint32_t level, uint64_t lo, uint64_t j,
+                                               uint64_t m) {
+  uint64_t h = splitmix64(splitmix64(splitmix64(seed ^ ((uint64_t)level << 56)) ^ lo) ^ j);
+  return __umul64hi(h, m);
+}
+
+// k_b rule: the paper's fixed k or the adaptive R29 rule.
+__device__ __host__ __forceinline__ uint32_t choose_kb(uint32_t k, uint32_t policy, uint32_t f, uint64_t M,
+                                                       uint64_t m) {
+  if (policy == 2) return k;
+  uint64_t want = (f * m + M - 1) / M;
+  uint32_t kb = 1;
+  while (kb < want && kb < k) kb <<= 1;
+  if (kb < 4) kb = 4;
+  if (kb > k) kb = k;
+  return kb;
+}
+
+__device__ __forceinline__ uint32_t ilog2(uint32_t x) { return 31 - __clz(x); }
+__device__ __forceinline__ uint32_t lanemask_lt() {
+  uint32_t r;
+  asm("mov.u32 %0, %%lanemask_lt;" : "=r"(r));
+  return r;
+}
+
+// --------------------------------------------------------------------------
+// Block-wide exclusive scan of one value per thread (NT threads).
+// --------------------------------------------------------------------------
+template <int NT>
+__device__ __forceinline__ uint32_t block_exclusive_scan(uint32_t x, uint32_t* s_warp, uint32_t* total) {
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  uint32_t inc = x;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    uint32_t y = __shfl_up_sync(kFull, inc, o);
+    if (lane >= o) inc += y;
+  }
+  if (lane == 31) s_warp[w] = inc;
+  __syncthreads();
+  if (w == 0) {
+    uint32_t v = lane < NT / 32 ? s_warp[lane] : 0;
+    uint32_t vi = v;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      uint32_t y = __shfl_up_sync(kFull, vi, o);
+      if (lane >= o) vi += y;
+    }
+    if (lane < NT / 32) s_warp[lane] = vi - v;
+    if (lane == NT / 32 - 1 && total) *total = vi;
+  }
+  __syncthreads();
+  uint32_t r = s_warp[w] + inc - x;
+  __syncthreads();
+  return r;
+}
+
+template <int NT>
+__device__ __forceinline__ uint64_t block_sum_u64(uint64_t x, unsigned long long* s_red) {
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(kFull, x, o);
+  if (lane == 0) s_red[w] = x;
+  __syncthreads();
+  uint64_t r = 0;
+#pragma unroll
+  for (int i = 0; i < NT / 32; i++) r += s_red[i];
+  __syncthreads();
+  return r;
+}
+
+// --------------------------------------------------------------------------
+// In-SM sort of up to NT*kItems keys (+ values) held in shared memory
+// (P:326-341): each thread sorts kItems keys with Batcher's odd-even merge
+// network [2], then log2(m / kItems) rounds of merge-path merges
+// through shared memory.  Shared layout: element i at i + i/16 (conflict-free
+// blocked access).
+// --------------------------------------------------------------------------
+__host__ __device__ constexpr int padded_len(int c) { return c + c / 16 + 1; }
+__device__ __forceinline__ int phys(int i) { return i + (i >> 4); }
+
+template <class Key, class Val, class Cmp>
+__device__ __forceinline__ void cmp_swap(Key& a, Key& b, Val& va, Val& vb, Cmp less) {
+  bool s = less(b, a);
+  Key lo = s ? b : a, hi = s ? a : b;
+  a = lo; b = hi;
+  if constexpr (kHasVal<Val>) {
+    Val l = s ? vb : va, h = s ? va : vb;
+    va = l; vb = h;
+  }
+}
+
+// Batcher odd-even merge sort network on k[LO .. LO+N), compile-time indices.
+template <int LO, int N, int R, class Key, class Val, class Cmp>
+__device__ __forceinline__ void oem_merge(Key* k, Val* v, Cmp less) {
+  constexpr int step = R * 2;
+  if constexpr (step < N) {
+    oem_merge<LO, N, step>(k, v, less);
+    oem_merge<LO + R, N, step>(k, v, less);
+#pragma unroll
+    for (int i = LO + R; i + R < LO + N; i += step) cmp_swap(k[i], k[i + R], v[i], v[i + R], less);
+  } else {
+    cmp_swap(k[LO], k[LO + R], v[LO], v[LO + R], less);
+  }
+}
+template <int LO, int N, class Key, class Val, class Cmp>
+__device__ __forceinline__ void oem_sort(Key* k, Val* v, Cmp less) {
+  if constexpr (N > 1) {
+    oem_sort<LO, N / 2>(k, v, less);
+    oem_sort<LO + N / 2, N / 2>(k, v, less);
+    oem_merge<LO, N, 1>(k, v, less);
+  }
+}
+
+// Stable odd-even transposition sort (only for the one partial thread).
+template <int N, class Key, class Val, class Cmp>
+__device__ __forceinline__ void transposition_sort(Key* k, Val* v, Cmp less) {
+#pragma unroll
+  for (int r = 0; r < N; r++) {
+#pragma unroll
+    for (int i = r & 1; i + 1 < N; i += 2) {
+      bool s = less(k[i + 1], k[i]);
+      Key a = s ? k[i + 1] : k[i], b = s ? k[i] : k[i + 1];
+      k[i] = a; k[i + 1] = b;
+      if constexpr (kHasVal<Val>) {
+        Val x = s ? v[i + 1] : v[i], y = s ? v[i] : v[i + 1];
+        v[i] = x; v[i + 1] = y;
+      }
+    }
+  }
+}
+
+template <class Key, class Val, int NT, class Cmp>
+struct CtaSort {
+  static constexpr int ITEMS = kItems;
+  static constexpr int C = NT * ITEMS;
+  static constexpr int PL = padded_len(C);
+  static constexpr size_t smem_bytes() {
+    return (size_t)PL * sizeof(Key) + (kHasVal<Val> ? (size_t)PL * sizeof(Val) : 0);
+  }
+
+  // Sorts sk[phys(0..m)) (and sv) in place; 0 <= m <= C.  Every thread of
+  // the NT-thread block must call it.  Begins and ends with a barrier.
+  __device__ static void sort(Key* sk, Val* sv, int m, Cmp less) {
+    __syncthreads();
+    const int t = threadIdx.x;
+    const int base = t * ITEMS;
+    const int cnt = min(max(m - base, 0), ITEMS);
+    Key k[ITEMS];
+    Val v[ITEMS];
+    if (cnt > 0) {
+#pragma unroll
+      for (int i = 0; i < ITEMS; i++) {
+        if (i < cnt) {
+          k[i] = sk[phys(base + i)];
+          if constexpr (kHasVal<Val>) v[i] = sv[phys(base + i)];
+        }
+      }
+      if (cnt == ITEMS) {
+        oem_sort<0, ITEMS>(k, v, less);
+      } else {
+        // pad with copies of the largest key; a stable network keeps the
+        // real keys ahead of the pads (which come last), so the first cnt
+        // outputs are exactly the real items
+        Key mx = k[0];
+#pragma unroll
+        for (int i = 1; i < ITEMS; i++)
+          if (i < cnt && less(mx, k[i])) mx = k[i];
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          if (i >= cnt) {
+            k[i] = mx;
+            if constexpr (kHasVal<Val>) v[i] = v[0];
+          }
+        }
+        transposition_sort<ITEMS>(k, v, less);
+      }
+#pragma unroll
+      for (int i = 0; i < ITEMS; i++) {
+        if (i < cnt) {
+          sk[phys(base + i)] = k[i];
+          if constexpr (kHasVal<Val>) sv[phys(base + i)] = v[i];
+        }
+      }
+    }
+    __syncthreads();
+    for (int w = ITEMS; w < m; w *= 2) {
+      if (cnt > 0) {
+        const int ps = (base / (2 * w)) * (2 * w);
+        const int a0 = ps, aLen = min(w, m - ps);
+        const int b0 = ps + w, bLen = max(0, min(w, m - ps - w));
+        const int diag = base - ps;
+        int lo = max(0, diag - bLen), hi = min(diag, aLen);
+        while (lo < hi) {                                  // merge path (stable: A first)
+          int mid = (lo + hi) >> 1;
+          Key a = sk[phys(a0 + mid)], b = sk[phys(b0 + diag - 1 - mid)];
+          if (less(b, a)) hi = mid; else lo = mid + 1;
+        }
+        int ai = lo, bi = diag - lo;
+        const int aLast = a0 + aLen - 1, bLast = b0 + max(bLen - 1, 0);
+        Key ka = sk[phys(min(a0 + ai, aLast))];
+        Key kb = sk[phys(min(b0 + bi, bLast))];
+        Val va, vb;
+        if constexpr (kHasVal<Val>) {
+          va = sv[phys(min(a0 + ai, aLast))];
+          vb = sv[phys(min(b0 + bi, bLast))];
+        }
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          bool takeA = (bi >= bLen) || (ai < aLen && !less(kb, ka));
+          k[i] = takeA ? ka : kb;
+          if constexpr (kHasVal<Val>) v[i] = takeA ? va : vb;
+          if (i + 1 < ITEMS) {
+            ai += takeA ? 1 : 0;
+            bi += takeA ? 0 : 1;
+            int idx = takeA ? min(a0 + ai, aLast) : min(b0 + bi, bLast);
+            Key x = sk[phys(idx)];
+            ka = takeA ? x : ka;
+            kb = takeA ? kb : x;
+            if constexpr (kHasVal<Val>) {
+              Val y = sv[phys(idx)];
+              va = takeA ? y : va;
+              vb = takeA ? vb : y;
+            }
+          }
+        }
+      }
+      __syncthreads();
+      if (cnt > 0) {
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          if (i < cnt) {
+            sk[phys(base + i)] = k[i];
+            if constexpr (kHasVal<Val>) sv[phys(base + i)] = v[i];
+          }
+        }
+      }
+      __syncthreads();
+    }
+  }
+};
+
+// --------------------------------------------------------------------------
+// Branch-free descent of the implicit splitter tree (Algorithm 2):
+// j := 1; repeat log k times j := 2j + (e > bt[j]); bucket = j - k.  The
+// comparison is less(bt[j], e) and becomes a predicated add.
+// --------------------------------------------------------------------------
+template <int LOGK, class Key, class Cmp>
+__device__ __forceinline__ uint32_t descend(const Key* __restrict__ tree, Key e, Cmp less) {
+  uint32_t j = 1;
+#pragma unroll
+  for (int d = 0; d < LOGK; d++) j = 2 * j + (less(tree[j], e) ? 1u : 0u);
+  return j - (1u << LOGK);
+}
+
+}  // namespace gss

@@ -1,0 +1,214 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle.
+
+Keys must match bit-exact; values (value = input index, R20) must form the
+same multiset of (key, value) pairs; one distribution level (gss_partition)
+must equal the oracle's stable partition, splitters and bucket sizes
+bit-exact (R7).
+"""
+import numpy as np
+import pytest
+import torch
+
+import inputs
+
+pytestmark = pytest.mark.gpu
+
+DT = {32: torch.uint32, 64: torch.uint64}
+
+
+@pytest.fixture(scope="module")
+def gss():
+    import paper_conf_ipps_leischneros10_b200 as g
+    g._lib()
+    return g
+
+
+def to_dev(a: np.ndarray) -> torch.Tensor:
+    return torch.from_numpy(np.ascontiguousarray(a)).cuda()
+
+
+def to_host(t: torch.Tensor) -> np.ndarray:
+    return t.cpu().numpy()
+
+
+def oracle_params(oracle_mod, k=256, M=16384, a=30, seed=5489, k_policy="adaptive", fill_div=4):
+    return oracle_mod.Params(k=k, a=a, M=M, k_policy=1 if k_policy == "adaptive" else 0, fill_div=fill_div,
+                             sample_cap=16384, seed=seed)
+
+
+def check_pairs(x, v_out, k_out):
+    n = x.size
+    vo = v_out.astype(np.int64)
+    np.testing.assert_array_equal(np.sort(vo), np.arange(n))
+    np.testing.assert_array_equal(x[vo], k_out)
+
+
+# ---------------------------------------------------------------------------
+# One level: gss_partition == oracle.distribute (a2..a6 bit-exact)
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("width", [32, 64])
+@pytest.mark.parametrize("dist", ["uniform", "dd", "and4", "sorted", "staggered", "equal"])
+@pytest.mark.parametrize("with_vals", [False, True])
+def test_partition_level_bit_exact(gss, oracle_mod, width, dist, with_vals):
+    n = 5 * 2048 * 3 + 777                                  # several tiles and a ragged tail
+    x = inputs.keys(dist, n, width, seed=3)
+    v = inputs.values(n, width) if with_vals else None
+    prm = dict(k=128, a=30, seed=77, k_policy="fixed", tile=2048)
+    ko, vo, spl, off, info = gss.partition(to_dev(x), to_dev(v) if with_vals else None, **prm)
+    ok, ov, rec = oracle_mod.distribute(x, v, oracle_params(oracle_mod, k=128, seed=77, k_policy="fixed", M=0))
+    assert info == (rec.kb, rec.ks, rec.eq, rec.K)
+    np.testing.assert_array_equal(to_host(spl).astype(np.uint64), rec.splitters)
+    np.testing.assert_array_equal(to_host(off).astype(np.uint64),
+                                  np.concatenate([[0], np.cumsum(rec.children)]).astype(np.uint64))
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if with_vals:
+        np.testing.assert_array_equal(to_host(vo), ov)
+
+
+# ---------------------------------------------------------------------------
+# Whole sort: keys bit-exact vs the oracle, values as a multiset
+# ---------------------------------------------------------------------------
+KINDS = [(32, False), (64, False), (32, True), (64, True)]
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist", inputs.DISTRIBUTIONS)
+def test_sort_distributions(gss, oracle_mod, width, pairs, dist):
+    n = (1 << 20) + 4321
+    x = inputs.keys(dist, n, width, seed=1)
+    v = inputs.values(n, width) if pairs else None
+    M = 4096
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=M, stats=True)
+    torch.cuda.synchronize()
+    assert st.error_flags == 0
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=M), log=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if pairs:
+        check_pairs(x, to_host(vo), ok)
+    # the level structure matches the oracle's records: keys split per level
+    for lvl in range(4):
+        want = sum(r.m for r in recs if r.level == lvl)
+        assert st.split_elems[lvl] == want, (lvl, st.split_elems[:4])
+    assert st.overflow_buckets == 0
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+def test_edge_sizes(gss, oracle_mod, width, pairs):
+    M = 16384 if not (pairs and width == 64) else 8192
+    for n in (0, 1, 2, 31, 32, 33, 2047, 2048, 2049, M - 1, M, M + 1, 3 * M + 5, 1 << 16):
+        x = inputs.keys("uniform", n, width, seed=n + 1)
+        v = inputs.values(n, width) if pairs else None
+        ko, vo = gss.sort(to_dev(x), to_dev(v) if pairs else None)
+        np.testing.assert_array_equal(to_host(ko), np.sort(x), err_msg=f"n={n}")
+        if pairs:
+            check_pairs(x, to_host(vo), np.sort(x))
+
+
+@pytest.mark.parametrize("k,policy", [(2, "fixed"), (4, "fixed"), (128, "fixed"), (1024, "fixed"), (512, "adaptive")])
+def test_k_values(gss, oracle_mod, k, policy):
+    n = 300_000
+    x = inputs.keys("gaussian", n, 64, seed=k)
+    M = 2048
+    ko, _, st = gss.sort(to_dev(x), k=k, M=M, k_policy=policy, stats=True)
+    assert st.error_flags == 0
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, k=k, M=M, k_policy=policy), log=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if st.overflow_buckets == 0:
+        for lvl in range(3):
+            assert st.split_elems[lvl] == sum(r.m for r in recs if r.level == lvl)
+
+
+def test_c1_config(gss, oracle_mod):
+    """BASELINE configs[0]: 2^16 uniform u32, k=128, one level + small sort."""
+    n = 1 << 16
+    x = inputs.keys("uniform", n, 32, seed=1)
+    ko, _, st = gss.sort(to_dev(x), k=128, k_policy="fixed", M=1 << 14, stats=True)
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, k=128, M=1 << 14, k_policy="fixed"), log=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    assert st.levels == 1 and len(recs) == 1
+    assert st.small_buckets == 128
+
+
+def test_overflow_fallback(gss, oracle_mod):
+    n = 1 << 18
+    for pairs in (False, True):
+        x = inputs.keys("uniform", n, 64, seed=4)
+        v = inputs.values(n, 64) if pairs else None
+        ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, k=16, k_policy="fixed", M=2048,
+                              max_levels=1, stats=True)
+        assert st.overflow_buckets > 0 and st.error_flags == 0
+        np.testing.assert_array_equal(to_host(ko), np.sort(x))
+        if pairs:
+            check_pairs(x, to_host(vo), np.sort(x))
+
+
+def test_in_place_and_descending(gss):
+    n = 200_003
+    x = inputs.keys("and2", n, 64, seed=5)
+    t = to_dev(x)
+    gss.sort(t, out=t)
+    np.testing.assert_array_equal(to_host(t), np.sort(x))
+    kd, _ = gss.sort(to_dev(x), descending=True)
+    np.testing.assert_array_equal(to_host(kd), np.sort(x)[::-1])
+    v = inputs.values(n, 64)
+    tk, tv = to_dev(x), to_dev(v)
+    gss.sort(tk, tv, out=tk, values_out=tv)
+    check_pairs(x, to_host(tv), np.sort(x))
+
+
+def test_sort_host_end_to_end(gss):
+    n = 1 << 20
+    for width, pairs in KINDS:
+        x = inputs.keys("uniform", n, width, seed=6)
+        hk = torch.from_numpy(x).pin_memory()
+        hv = torch.from_numpy(inputs.values(n, width)).pin_memory() if pairs else None
+        ko, vo = gss.sort_host(hk, hv)
+        np.testing.assert_array_equal(ko.numpy(), np.sort(x))
+        if pairs:
+            check_pairs(x, vo.numpy(), np.sort(x))
+
+
+def test_partition_by_and_sample(gss, oracle_mod):
+    n = 123_457
+    x = inputs.keys("uniform", n, 64, seed=8)
+    v = inputs.values(n, 64)
+    spl = np.sort(x[[5, 99, 1000, 5000, 77777, 100000, 120000]])
+    ko, vo, cnt = gss.partition_by(to_dev(x), to_dev(v), to_dev(spl))
+    ids = np.searchsorted(spl, x, side="left")              # #{spl < e}, ties go left
+    order = np.argsort(ids, kind="stable")
+    np.testing.assert_array_equal(to_host(ko), x[order])
+    np.testing.assert_array_equal(to_host(vo), v[order])
+    np.testing.assert_array_equal(to_host(cnt), np.bincount(ids, minlength=len(spl) + 1))
+    s = gss.sample(to_dev(x), 1000, lo_global=12345, level_tag=255, seed=9)
+    want = [x[(oracle_mod.sample_hash(9, 255, 12345, j) * n) >> 64] for j in range(1000)]
+    np.testing.assert_array_equal(to_host(s), np.array(want, dtype=np.uint64))
+
+
+def test_deterministic(gss):
+    n = 1 << 20
+    x = inputs.keys("dd", n, 64)
+    v = inputs.values(n, 64)
+    a = gss.sort(to_dev(x), to_dev(v))
+    b = gss.sort(to_dev(x), to_dev(v))
+    assert torch.equal(a[0], b[0]) and torch.equal(a[1], b[1])
+
+
+# ---------------------------------------------------------------------------
+# BASELINE sizes, in the configuration bench.py times: properties at any size
+# plus sampled ranks computed one by one by the oracle.
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("width,n,dist", [(64, 1 << 28, "uniform"), (32, 1 << 27, "uniform"),
+                                          (32, 1 << 27, "dd"), (64, 1 << 27, "and4")])
+def test_full_size(gss, oracle_mod, width, n, dist):
+    x = inputs.keys(dist, n, width, seed=1)
+    ko, _, st = gss.sort(to_dev(x), stats=True)
+    assert st.error_flags == 0
+    y = to_host(ko)
+    assert np.all(y[1:] >= y[:-1])                          # non-decreasing
+    # same multiset: order-independent sums of a mixing function
+    def mix(a):
+        z = a.astype(np.uint64) * np.uint64(0x9E3779B97F4A7C15)
+        return np.bitwise_xor.reduce(z ^ (z >> np.uint64(29))), int(a.astype(np.uint64).sum(dtype=np.uint64))
+    assert mix(x) == mix(y)
+    for r in (0, n // 3, n - 1):
+        assert int(y[r]) == oracle_mod.select(x, r)
