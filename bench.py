@@ -1,0 +1,359 @@
+#!/usr/bin/env python3
+"""Benchmark of the B200 GPU sample sort (BASELINE.json metric: Gkeys/s and % of
+the HBM roofline).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+                    [--workload c4_u64_2p28|c2_u32_2p27|c3_u64_2p27|c3_kv64_2p27|c1_u32_2p16]
+
+One step = one full sort (every level of the k-way distribution pass plus the
+in-SM bucket sorts) of the workload's synthetic input, already resident in HBM
+(host<->device transfer excluded as in the paper).  Inputs are larger
+than the 126 MB L2 (except C1, which is latency-bound and says so).  N > 1
+runs under torchrun, one process per GPU: the distributed sample sort
+(paper_conf_ipps_leischneros10_b200.dist) with weak scaling (n keys per GPU).
+Rank 0 prints one JSON line.
+
+--impl reference times the CPU oracle (oracle/, the plain sample sort written
+from the paper) on the host cores on a bounded sample of the same workload.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import subprocess
+import sys
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import inputs  # noqa: E402
+
+WORKLOADS = {
+    # name: (n, key bits, pairs, distribution, description)
+    "c4_u64_2p28": (1 << 28, 64, False, "uniform", "2^28 uniform u64 keys (BASELINE configs[3], the north-star target row)"),
+    "c2_u32_2p27": (1 << 27, 32, False, "uniform", "2^27 uniform u32 keys (BASELINE configs[1])"),
+    "c3_u64_2p27": (1 << 27, 64, False, "uniform", "2^27 uniform u64 keys (BASELINE configs[2])"),
+    "c3_kv64_2p27": (1 << 27, 64, True, "uniform", "2^27 uniform u64 key + u64 value pairs (BASELINE configs[2])"),
+    "c1_u32_2p16": (1 << 16, 32, False, "uniform", "2^16 uniform u32 keys, k=128 (BASELINE configs[0]; launch-bound)"),
+}
+DEFAULT_WORKLOAD = "c4_u64_2p28"
+CPU_SAMPLE_N = 1 << 26
+
+
+def peaks():
+    path = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(path):
+        d = json.load(open(path))
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs: torch copy_, read+write)"
+    return 6650.0, "fallback (B200_PROFILING.md: 6.65 TB/s)"
+
+
+def alg_bytes(kind: str, st, wk: int, wv: int, k: int, T: int, a: int, steps: int = 1) -> float:
+    """Algorithmic bytes per step of one kernel kind."""
+    split = sum(st.split_elems)
+    if kind == "classify":
+        return split * wk                                     # Phase 2 reads every key once
+    if kind == "scatter":
+        return split * (2 * wk + 2 * wv)                      # Phase 4 reads and writes key + value
+    if kind == "small_sort":
+        return st.small_elems * 2 * (wk + wv)                 # one read, one write
+    if kind == "scan":
+        return split * 16.0 * k / T                           # histogram written, scanned (r+w), read
+    if kind == "sample":
+        return sum(st.split_buckets) * a * k * 32             # one sector per sampled key
+    if kind == "copy":
+        return st.eq_elems * 2 * (wk + wv)
+    return 0.0
+
+
+def total_alg_bytes(st, wk, wv, k, T, a):
+    return sum(alg_bytes(x, st, wk, wv, k, T, a) for x in ("classify", "scatter", "small_sort", "scan", "sample", "copy"))
+
+
+class ClockSampler:
+    """nvidia-smi clocks and throttle reasons sampled during the timed region."""
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
+         "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+         "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.p = None
+
+    def __enter__(self):
+        try:
+            self.p = subprocess.Popen(["nvidia-smi", f"--query-gpu={self.Q}", "--format=csv,noheader,nounits",
+                                       "-lms", "100", "-i", str(self.index)], stdout=subprocess.PIPE,
+                                      stderr=subprocess.DEVNULL, text=True)
+        except Exception:
+            self.p = None
+        time.sleep(0.3)
+        return self
+
+    def __exit__(self, *a):
+        self.out = ""
+        if self.p is not None:
+            time.sleep(0.2)
+            self.p.terminate()
+            try:
+                self.out, _ = self.p.communicate(timeout=5)
+            except Exception:
+                self.p.kill()
+                self.out = ""
+
+    def summary(self):
+        rows = []
+        for line in (self.out or "").strip().splitlines():
+            f = [x.strip() for x in line.split(",")]
+            if len(f) >= 7:
+                try:
+                    rows.append((float(f[0]), float(f[1]), f[2:]))
+                except ValueError:
+                    pass
+        if not rows:
+            return None
+        sm = [r[0] for r in rows]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in rows for i, v in enumerate(r[2][1:5]) if v.lower() == "active"})
+        load = [s for s in sm if s > 0.5 * max(sm)]
+        return {"sm_mhz": float(np.median(load or sm)), "sm_max_mhz": max(r[1] for r in rows), "reasons": reasons,
+                "samples": len(rows)}
+
+
+def mix_check(x: np.ndarray, y: np.ndarray) -> bool:
+    """Order-independent multiset fingerprint + sortedness (result check, not timed)."""
+    if not np.all(y[1:] >= y[:-1]):
+        return False
+    def fp(a):
+        z = a.astype(np.uint64) * np.uint64(0x9E3779B97F4A7C15)
+        return int(np.bitwise_xor.reduce(z ^ (z >> np.uint64(29)))), int(a.astype(np.uint64).sum(dtype=np.uint64))
+    return fp(x) == fp(y)
+
+
+# ---------------------------------------------------------------------------
+# reference arm: the CPU oracle
+# ---------------------------------------------------------------------------
+def run_reference(args, wl):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return 0
+    import oracle
+    oracle.build()
+    n, bits, pairs, dist, desc = WORKLOADS[wl]
+    ns = min(n, CPU_SAMPLE_N)
+    x = inputs.keys(dist, ns, bits, seed=1) if dist != "sorted" else inputs.keys(dist, ns, bits)
+    v = inputs.values(ns, bits) if pairs else None
+    prm = oracle.Params(k=256, a=30, M=8192 if (pairs and bits == 64) else 16384, k_policy=1, fill_div=4, seed=5489)
+    if wl == "c1_u32_2p16":
+        prm.k, prm.k_policy = 128, 0
+    times = []
+    for i in range(args.warmup + args.steps):
+        t0 = time.perf_counter()
+        oracle.sort(x, v, prm)
+        t1 = time.perf_counter()
+        if i >= args.warmup:
+            times.append(t1 - t0)
+    t = float(np.mean(times))
+    val = ns / t / 1e9
+    line = {
+        "impl": "reference", "metric": f"sorting rate (Gkeys/s, {'pairs' if pairs else 'keys'})", "value": val,
+        "unit": "Gkeys/s", "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+        "ms_per_step": t * 1e3, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+        "dtype": f"u{bits}", "data": "synthetic",
+        "config": {"workload": wl, "description": desc, "n_sample": ns, "dist": dist},
+        "cpu_baseline": {"value": val, "unit": "Gkeys/s", "cores": 1, "kind": "oracle",
+                         "sample": f"first {ns} keys of the workload's generator ({dist}, seed 1), one thread"},
+        "e2e": {"value": val, "unit": "Gkeys/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+# ---------------------------------------------------------------------------
+# our arm
+# ---------------------------------------------------------------------------
+def run_ours(args, wl):
+    import torch
+    import torch.distributed as dist_mod
+
+    import paper_conf_ipps_leischneros10_b200 as gss
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        dist_mod.init_process_group("nccl", device_id=dev)
+
+    n, bits, pairs, distname, desc = WORKLOADS[wl]
+    wk = bits // 8
+    wv = wk if pairs else 0
+    kind = f"u{bits}"
+    params = dict(k=256, a=30, tile=16384)
+    if wl == "c1_u32_2p16":
+        params.update(k=128, k_policy="fixed")
+    M = 8192 if (pairs and bits == 64) else 16384
+    params["M"] = M
+
+    # input: this rank's shard of the global input (weak scaling: n keys per GPU)
+    x = inputs.keys(distname, n * world, bits, seed=1, start=rank * n, count=n)
+    hv = inputs.values(n, bits, start=rank * n) if pairs else None
+    dkeys = torch.from_numpy(x).to(dev)
+    dvals = torch.from_numpy(hv).to(dev) if pairs else None
+    stream = torch.cuda.current_stream(dev)
+
+    if world > 1:
+        from paper_conf_ipps_leischneros10_b200 import dist as gdist
+        sorter = gdist.DistSorter(kind, n, pairs, device=dev, **params)
+        step = lambda: sorter(dkeys, dvals)  # noqa: E731
+    else:
+        sorter = gss.Sorter(kind, n, pairs, device=dev, **params)
+        kout = torch.empty_like(dkeys)
+        vout = torch.empty_like(dvals) if pairs else None
+        step = lambda: sorter(dkeys, kout, dvals, vout)  # noqa: E731
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize(dev)
+
+    def barrier():
+        if world > 1:
+            dist_mod.barrier()
+
+    with ClockSampler(local) as clk:
+        barrier()
+        torch.cuda.synchronize(dev)
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        for _ in range(args.steps):
+            step()
+        e1.record(stream)
+        torch.cuda.synchronize(dev)
+        barrier()
+    ms = e0.elapsed_time(e1) / args.steps
+    if world > 1:
+        t = torch.tensor([ms], device=dev, dtype=torch.float64)
+        dist_mod.all_reduce(t, op=dist_mod.ReduceOp.MAX)
+        ms = float(t.item())
+    value = n * world / (ms * 1e-3) / 1e9
+
+    # ---- result check (not timed) ----
+    if world == 1:
+        ok = mix_check(x, kout.cpu().numpy())
+    else:
+        ok = sorter.verify(x)
+
+    # ---- per-kernel breakdown (separate profiled steps, CUDA events per launch) ----
+    extra = {}
+    roof = None
+    gpu_launches = None
+    hbm, peak_src = peaks()
+    if world == 1:
+        st = sorter(dkeys, kout, dvals, vout, stats=True)
+        gpu_launches = st.launches * args.steps
+        prof = gss.Profiler()
+        kp = max(3, min(args.steps, 10))
+        for _ in range(kp):
+            sorter(dkeys, kout, dvals, vout, profiler=prof)
+        torch.cuda.synchronize(dev)
+        per = {k: (v[0] / kp, v[1] / kp) for k, v in prof.read().items() if v[1]}
+        kernels_ms = {k: round(v[0], 4) for k, v in per.items()}
+        dom = max((k for k in per if k not in ("h2d", "d2h")), key=lambda k: per[k][0])
+        a = params["a"]
+        ab = alg_bytes(dom, st, wk, wv, params["k"], params["tile"], a)
+        achieved = ab / (per[dom][0] * 1e-3) / 1e9
+        traffic = None
+        tpath = os.path.join(ROOT, "profiles", f"ncu_traffic_{wl}.json")
+        if os.path.exists(tpath):
+            tr = json.load(open(tpath))
+            if dom in tr:
+                traffic = tr[dom]
+        roof = {"bound": "hbm", "kernel": dom, "achieved": round(achieved, 1), "peak": hbm, "unit": "GB/s",
+                "frac": round(achieved / hbm, 4), "traffic": traffic, "alg_bytes_per_step": ab,
+                "launches_per_step": per[dom][1], "peak_source": peak_src}
+        B = total_alg_bytes(st, wk, wv, params["k"], params["tile"], a)
+        extra["kernels_ms_per_step"] = kernels_ms
+        extra["whole_sort_roofline"] = {"alg_bytes": B, "t_roof_ms": B / (hbm * 1e9) * 1e3,
+                                        "frac": round(B / (hbm * 1e9) / (ms * 1e-3), 4),
+                                        "levels": st.levels, "split_elems": st.split_elems[: max(st.levels, 1)],
+                                        "small_buckets": st.small_buckets}
+    # ---- end to end through the C ABI with host buffers ----
+    e2e = None
+    if world == 1:
+        hs = gss.HostSorter(kind, n, pairs, device=dev, **params)
+        hk = torch.from_numpy(x).pin_memory()
+        ho = torch.empty_like(hk).pin_memory()
+        hvi = torch.from_numpy(hv).pin_memory() if pairs else None
+        hvo = torch.empty_like(hvi).pin_memory() if pairs else None
+        for _ in range(2):
+            hs(hk, ho, hvi, hvo)
+        torch.cuda.synchronize(dev)
+        ke = max(2, min(args.steps, 5))
+        e0.record(stream)
+        for _ in range(ke):
+            hs(hk, ho, hvi, hvo)
+        e1.record(stream)
+        torch.cuda.synchronize(dev)
+        ems = e0.elapsed_time(e1) / ke
+        ok = ok and bool(np.array_equal(ho.numpy(), kout.cpu().numpy()))
+        e2e = {"value": n / (ems * 1e-3) / 1e9, "unit": "Gkeys/s", "h2d_bytes_per_step": n * (wk + wv),
+               "d2h_bytes_per_step": n * (wk + wv), "ms_per_step": ems}
+
+    # ---- CPU baseline: the oracle on a bounded sample (rank 0, N == 1 only) ----
+    cpu = None
+    if world == 1 and not args.no_cpu_baseline:
+        import oracle
+        oracle.build()
+        ns = min(n, CPU_SAMPLE_N)
+        xs = x[:ns] if distname != "sorted" else inputs.keys(distname, ns, bits)
+        vs = hv[:ns] if pairs else None
+        prm = oracle.Params(k=params["k"], a=30, M=M, k_policy=0 if params.get("k_policy") == "fixed" else 1,
+                            fill_div=4, seed=5489)
+        t0 = time.perf_counter()
+        oracle.sort(xs, vs, prm)
+        ct = time.perf_counter() - t0
+        cpu = {"value": ns / ct / 1e9, "unit": "Gkeys/s", "cores": 1, "kind": "oracle",
+               "sample": f"first {ns} keys of this workload's input, one oracle sort on one host thread ({ct:.1f} s)"}
+
+    if rank == 0:
+        line = {
+            "metric": f"sorting rate (Gkeys/s, {'key-value pairs' if pairs else 'keys'}); % HBM roofline",
+            "value": round(value, 3), "unit": "Gkeys/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": round(ms, 4), "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": kind, "data": "synthetic",
+            "config": {"workload": wl, "description": desc, "n_per_gpu": n, "dist": distname, "key": kind,
+                       "values": kind if pairs else None, **{k: v for k, v in params.items()},
+                       "l2": "inputs larger than the 126 MB L2" if n * wk > (256 << 20) else
+                       "input fits in L2 (latency-bound config)", "parallelism": f"dp{world}"},
+            "roofline": roof, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": gpu_launches,
+            "clocks": clk.summary(), "result_check": bool(ok), **extra,
+        }
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        dist_mod.destroy_process_group()
+    return 0 if ok else 1
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--workload", default=DEFAULT_WORKLOAD, choices=sorted(WORKLOADS))
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    args = ap.parse_args()
+    if args.warmup < 3 and args.impl == "ours":
+        args.warmup = 3
+    if args.impl == "reference":
+        return run_reference(args, args.workload)
+    return run_ours(args, args.workload)
+
+
+if __name__ == "__main__":
+    sys.exit(main())

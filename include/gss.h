@@ -102,7 +102,9 @@ typedef struct gss_params {
 } gss_params;
 
 #define GSS_FLAG_RECOMPUTE_IDS 1u  /* Phase 4 re-descends the tree instead of reading stored
-                                      bucket ids (the paper's choice)            */
+                                      bucket ids (the paper's choice); reserved  */
+#define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets with one more sample-sort split inside
+                                      shared memory + warp merge sorts (P:332-335 variant)  */
 
 /* Human-readable name of a status code (static storage). */
 const char* gss_status_string(gss_status s);

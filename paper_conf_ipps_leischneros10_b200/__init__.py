@@ -19,7 +19,7 @@ import torch
 
 from . import _build
 
-__all__ = ["sort", "sort_host", "partition", "partition_by", "sample", "Profiler", "Stats", "temp_bytes",
+__all__ = ["sort", "sort_host", "Sorter", "HostSorter", "partition", "partition_by", "sample", "Profiler", "Stats", "temp_bytes",
            "library_path", "KERNEL_KINDS"]
 
 KERNEL_KINDS = ["init", "sample", "classify", "scan", "scatter", "plan", "small_sort", "copy", "overflow", "h2d",
@@ -255,6 +255,37 @@ def temp_bytes(kind: str, n: int, pairs: bool = False, host: bool = False, **par
         rc = fn(None, None, n, None, ctypes.byref(tb), None, ctypes.byref(p))
     _check(rc, fn.__name__)
     return tb.value
+
+
+class Sorter:
+    """Repeated device sorts of n keys (and values) with a persistent scratch
+    buffer: the call a benchmark or a serving loop makes."""
+
+    def __init__(self, kind: str, n: int, pairs: bool = False, device=None, descending: bool = False, **params):
+        self.lib = _lib()
+        self.kind, self.n, self.pairs = kind, n, pairs
+        self.device = torch.device(device or "cuda")
+        self.params = params
+        self.temp = torch.empty(max(temp_bytes(kind, n, pairs, **params), 1), dtype=torch.uint8, device=self.device)
+        if descending:
+            if pairs or kind != "u64":
+                raise NotImplementedError("descending order is exported for keys-only u64")
+            self.fn = self.lib.gss_sort_u64_descending
+        else:
+            self.fn = getattr(self.lib, f"gss_sort_{'pairs_' if pairs else ''}{kind}")
+
+    def __call__(self, keys, out, vals=None, vals_out=None, stream=None, profiler=None, stats=False):
+        st = _Stats() if stats else None
+        p = _params(stats=st, profiler=profiler, **self.params)
+        s = stream.cuda_stream if stream is not None else torch.cuda.current_stream(self.device).cuda_stream
+        tb = _sz(self.temp.numel())
+        if self.pairs:
+            rc = self.fn(_ptr(keys), _ptr(vals), _ptr(out), _ptr(vals_out), self.n, _ptr(self.temp),
+                         ctypes.byref(tb), s, ctypes.byref(p))
+        else:
+            rc = self.fn(_ptr(keys), _ptr(out), self.n, _ptr(self.temp), ctypes.byref(tb), s, ctypes.byref(p))
+        _check(rc, self.fn.__name__)
+        return Stats._from(st) if stats else None
 
 
 class HostSorter:

@@ -32,7 +32,6 @@ namespace {
 
 constexpr uint32_t kVersion = 1;
 constexpr uint32_t kClassCap[kNumClasses] = {2048, 4096, 8192, 16384};
-constexpr uint32_t kClassThreads[kNumClasses] = {128, 256, 512, 1024};
 
 size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -118,6 +117,7 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
 template <class Key, class Val, class IdT>
 struct Layout {
   size_t off_cnt, off_ktmp, off_vtmp, off_ids, off_bk[2], off_tb[2], off_hist[2], off_spl[2], off_small[kNumClasses],
+      off_retry[kNumClasses],
       off_copy, off_ovf, off_scan, off_hin_k, off_hin_v, off_hout_k, off_hout_v, total;
   uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_small[kNumClasses];
 
@@ -157,6 +157,7 @@ struct Layout {
       off_spl[s] = take((size_t)cap_spl * sizeof(Key));
     }
     for (int i = 0; i < kNumClasses; i++) off_small[i] = take((size_t)cap_small[i] * sizeof(Item));
+    for (int i = 0; i < kNumClasses; i++) off_retry[i] = take((size_t)cap_small[i] * sizeof(Item));
     off_copy = take((size_t)cap_copy * sizeof(Item));
     off_ovf = take((size_t)cap_ovf * sizeof(Item));
     off_scan = take(kScanCtas * 4);
@@ -192,6 +193,8 @@ gss_status launch(gss_profiler* prof, int kind, cudaStream_t s, uint32_t* count,
   return e == cudaSuccess ? GSS_SUCCESS : GSS_ERROR_CUDA;
 }
 
+// Opt in to the dynamic shared memory a kernel needs and ask for the largest
+// shared-memory carveout, so that several CTAs share an SM.
 template <class K>
 gss_status set_smem(K kernel, size_t bytes) {
   if (bytes > 48 * 1024) {
@@ -199,6 +202,11 @@ gss_status set_smem(K kernel, size_t bytes) {
       cudaGetLastError();
       return GSS_ERROR_CUDA;
     }
+  }
+  if (cudaFuncSetAttribute(kernel, cudaFuncAttributePreferredSharedMemoryCarveout, cudaSharedmemCarveoutMaxShared) !=
+      cudaSuccess) {
+    cudaGetLastError();
+    return GSS_ERROR_CUDA;
   }
   return GSS_SUCCESS;
 }
@@ -237,6 +245,7 @@ struct Engine {
     }
     for (int i = 0; i < kNumClasses; i++) {
       c.small[i] = reinterpret_cast<Item*>(base + lay.off_small[i]);
+      c.retry[i] = reinterpret_cast<Item*>(base + lay.off_retry[i]);
       c.cap_small[i] = lay.cap_small[i];
       c.class_cap[i] = cfg.class_cap[i];
     }
@@ -255,15 +264,43 @@ struct Engine {
     return c;
   }
 
-  template <int NT>
+  template <int CAP>
   static gss_status launch_small(C& c, const Cfg& cfg, int cls, const DeviceInfo& di, cudaStream_t s,
-                                 gss_profiler* prof, uint32_t* count) {
-    auto kern = k_small<Key, Val, IdT, Cmp, NT>;
+                                 gss_profiler* prof, uint32_t* count, uint32_t retry) {
+    constexpr int NT = small_threads<Key, Val, CAP>();
+    auto kern = k_small<Key, Val, IdT, Cmp, CAP>;
     const size_t smem = CtaSort<Key, Val, NT, Cmp>::smem_bytes();
     GSS_TRY(set_smem(kern, smem));
     static int grid = 0;
     if (!grid) grid = grid_for(kern, NT, smem, di.sms);
+    return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<grid, NT, smem, s>>>(c, (uint32_t)cls, retry); });
+  }
+
+  template <int CAP>
+  static gss_status launch_split(C& c, const Cfg& cfg, int cls, const DeviceInfo& di, cudaStream_t s,
+                                 gss_profiler* prof, uint32_t* count) {
+    constexpr int NT = split_threads<Key, Val, CAP>();
+    auto kern = k_split_sort<Key, Val, IdT, Cmp, CAP>;
+    const size_t smem = SplitSortSmem<Key, Val, CAP, NT>::bytes();
+    GSS_TRY(set_smem(kern, smem));
+    static int grid = 0;
+    if (!grid) grid = grid_for(kern, NT, smem, di.sms);
     return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<grid, NT, smem, s>>>(c, (uint32_t)cls); });
+  }
+
+  template <int CAP>
+  static gss_status launch_class(C& c, const Cfg& cfg, int cls, const DeviceInfo& di, cudaStream_t s,
+                                 gss_profiler* prof, uint32_t* count, int phase) {
+    // phase 0: the bucket lists; phase 1: the retry lists (sub-buckets an
+    // in-SM split could not finish).  The in-SM sample split (k_split_sort) is
+    // built but not selected: on B200 its warp-level sub-bucket sorts cost more
+    // than the block-wide merge sort (profiles/r01 notes).
+    if (cfg.flags & GSS_FLAG_SPLIT_SORT) {
+      if (phase == 0) return launch_split<CAP>(c, cfg, cls, di, s, prof, count);
+      return launch_small<CAP>(c, cfg, cls, di, s, prof, count, 1u);
+    }
+    if (phase == 0) return launch_small<CAP>(c, cfg, cls, di, s, prof, count, 0u);
+    return GSS_SUCCESS;
   }
 
   // The whole launch sequence.  mode: sort / partition / partition_by.
@@ -277,7 +314,7 @@ struct Engine {
     auto kc = k_classify<Key, Val, IdT, Cmp>;
     const size_t sm_cls = (size_t)kmax * sizeof(Key) * 2 + (size_t)(kClsThreads / 32) * kmax * 4;
     auto ksc = k_scatter<Key, Val, IdT, Cmp>;
-    const size_t sm_sc = ScatterSmem<Key, Val>::bytes(kmax);
+    const size_t sm_sc = ScatterSmem<Key, Val, IdT>::bytes(kmax);
     GSS_TRY(set_smem(ks, sm_sample));
     GSS_TRY(set_smem(kc, sm_cls));
     GSS_TRY(set_smem(ksc, sm_sc));
@@ -303,20 +340,23 @@ struct Engine {
     }
     if (mode != MODE_SORT) return GSS_SUCCESS;
     // in-SM sorts, largest class first (buckets "ordered by size"; R8)
-    for (int cls = (int)cfg.nclass - 1; cls >= 0; cls--) {
-      switch (kClassThreads[cls]) {
-        case 128: GSS_TRY(launch_small<128>(c, cfg, cls, di, s, prof, count)); break;
-        case 256: GSS_TRY(launch_small<256>(c, cfg, cls, di, s, prof, count)); break;
-        case 512: GSS_TRY(launch_small<512>(c, cfg, cls, di, s, prof, count)); break;
-        case 1024:
-          if constexpr (max_small_capacity<Key, Val>() >= 16384) {
-            GSS_TRY(launch_small<1024>(c, cfg, cls, di, s, prof, count));
-          }
-          break;
+    // phase 0: in-SM sample split + warp sorts; phase 1: block merge sort of the retries
+    for (int phase = 0; phase < 2; phase++) {
+      for (int cls = (int)cfg.nclass - 1; cls >= 0; cls--) {
+        switch (kClassCap[cls]) {
+          case 2048: GSS_TRY(launch_class<2048>(c, cfg, cls, di, s, prof, count, phase)); break;
+          case 4096: GSS_TRY(launch_class<4096>(c, cfg, cls, di, s, prof, count, phase)); break;
+          case 8192: GSS_TRY(launch_class<8192>(c, cfg, cls, di, s, prof, count, phase)); break;
+          case 16384:
+            if constexpr (max_small_capacity<Key, Val>() >= 16384) {
+              GSS_TRY(launch_class<16384>(c, cfg, cls, di, s, prof, count, phase));
+            }
+            break;
+        }
       }
     }
     GSS_TRY(launch(prof, GSS_K_COPY, s, count, [&] { k_copy<Key, Val, IdT><<<di.sms * 4, 256, 0, s>>>(c); }));
-    constexpr int NTO = kHasVal<Val> && (sizeof(Key) + sizeof(Val) > 8) ? 512 : 1024;
+    constexpr int NTO = 1024;
     auto ko = k_overflow<Key, Val, IdT, Cmp, NTO>;
     const size_t sm_ovf = CtaSort<Key, Val, NTO, Cmp>::smem_bytes();
     GSS_TRY(set_smem(ko, sm_ovf));

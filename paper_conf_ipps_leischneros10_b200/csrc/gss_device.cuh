@@ -13,7 +13,6 @@ namespace gss {
 
 constexpr int kNumClasses = 4;        // in-SM sort size classes (2K, 4K, 8K, 16K keys)
 constexpr int kMaxLevels = 16;        // distribution levels launched at most
-constexpr int kItems = 16;            // keys per thread in the in-SM sort
 constexpr uint32_t kFull = 0xffffffffu;
 
 enum Buf : uint32_t { BUF_IN = 0, BUF_TMP = 1, BUF_OUT = 2 };
@@ -58,6 +57,7 @@ struct LevelCounters {
 struct Counters {
   LevelCounters lvl[kMaxLevels + 1];
   uint32_t small_count[kNumClasses];
+  uint32_t retry_count[kNumClasses];   // sub-buckets the in-SM sample split could not finish
   uint32_t copy_count, ovf_count, err, pad;
   unsigned long long small_elems, max_small, eq_buckets, eq_elems, ovf_elems;
 };
@@ -74,6 +74,7 @@ struct Ctx {
   uint32_t* hist[2];
   Key* spl[2];
   Item* small[kNumClasses];
+  Item* retry[kNumClasses];
   Item* copy;
   Item* ovf;
   uint32_t* scan_part;
@@ -241,20 +242,69 @@ __device__ __forceinline__ void transposition_sort(Key* k, Val* v, Cmp less) {
   }
 }
 
-template <class Key, class Val, int NT, class Cmp>
+// keys per thread of the in-SM sort: 16, or 8 for 16-byte pairs (register budget)
+template <class Key, class Val>
+constexpr int sort_items() {
+  return (kHasVal<Val> && sizeof(Key) + sizeof(Val) > 8) ? 8 : 16;
+}
+
+template <class Key, class Val, int NT, class Cmp, int ITEMS_ = sort_items<Key, Val>()>
 struct CtaSort {
-  static constexpr int ITEMS = kItems;
+  static constexpr int ITEMS = ITEMS_;
   static constexpr int C = NT * ITEMS;
   static constexpr int PL = padded_len(C);
   static constexpr size_t smem_bytes() {
     return (size_t)PL * sizeof(Key) + (kHasVal<Val> ? (size_t)PL * sizeof(Val) : 0);
   }
 
+  // Merge-path split of output diagonal `diag` of runs A = sk[a0, a0+aLen),
+  // B = sk[b0, b0+bLen) (stable: A first on ties), then ITEMS outputs into
+  // k/v.  One branch-free path: a run that is exhausted is never taken, and
+  // the element read one past its end lies inside the buffer and is unused.
+  __device__ static __forceinline__ void merge_items(const Key* sk, const Val* sv, int a0, int aLen, int b0,
+                                                     int bLen, int diag, Key* k, Val* v, Cmp less) {
+    int lo = max(0, diag - bLen), hi = min(diag, aLen);
+    while (lo < hi) {
+      const int mid = (lo + hi) >> 1;
+      if (less(sk[phys(b0 + diag - 1 - mid)], sk[phys(a0 + mid)])) hi = mid; else lo = mid + 1;
+    }
+    int ia = a0 + lo, ib = b0 + diag - lo;
+    const int ae = a0 + aLen, be = b0 + bLen;
+    Key ka = sk[phys(ia)], kb = sk[phys(ib)];
+    Val va, vb;
+    if constexpr (kHasVal<Val>) { va = sv[phys(ia)]; vb = sv[phys(ib)]; }
+#pragma unroll
+    for (int i = 0; i < ITEMS; i++) {
+      const bool p = (ib >= be) || (ia < ae && !less(kb, ka));
+      k[i] = p ? ka : kb;
+      if constexpr (kHasVal<Val>) v[i] = p ? va : vb;
+      if (i + 1 < ITEMS) {
+        const int nx = (p ? ia : ib) + 1;
+        const Key x = sk[phys(nx)];
+        ia = p ? nx : ia;
+        ib = p ? ib : nx;
+        ka = p ? x : ka;
+        kb = p ? kb : x;
+        if constexpr (kHasVal<Val>) {
+          const Val y = sv[phys(nx)];
+          va = p ? y : va;
+          vb = p ? vb : y;
+        }
+      }
+    }
+  }
+
+  // NT == 32: a single warp sorts on its own (only warp barriers).
+  __device__ static __forceinline__ void bar() {
+    if constexpr (NT == 32) __syncwarp(); else __syncthreads();
+  }
+
   // Sorts sk[phys(0..m)) (and sv) in place; 0 <= m <= C.  Every thread of
-  // the NT-thread block must call it.  Begins and ends with a barrier.
+  // the NT-thread block (or every lane of the warp when NT == 32) must call
+  // it.  Begins and ends with a barrier.
   __device__ static void sort(Key* sk, Val* sv, int m, Cmp less) {
-    __syncthreads();
-    const int t = threadIdx.x;
+    bar();
+    const int t = NT == 32 ? (threadIdx.x & 31) : threadIdx.x;
     const int base = t * ITEMS;
     const int cnt = min(max(m - base, 0), ITEMS);
     Key k[ITEMS];
@@ -267,24 +317,38 @@ struct CtaSort {
           if constexpr (kHasVal<Val>) v[i] = sv[phys(base + i)];
         }
       }
-      if (cnt == ITEMS) {
-        oem_sort<0, ITEMS>(k, v, less);
-      } else {
-        // pad with copies of the largest key; a stable network keeps the
-        // real keys ahead of the pads (which come last), so the first cnt
-        // outputs are exactly the real items
+      // A partial thread pads with copies of its largest item: after sorting,
+      // its first cnt outputs are exactly its real items because every pad is
+      // indistinguishable from that item (same key, and the same value for
+      // pairs).  Only pairs with a repeated largest key need the stable
+      // transposition network instead (pads last, real items first).
+      bool stable_path = false;
+      if (cnt < ITEMS) {
         Key mx = k[0];
+        Val vmx = v[0];
 #pragma unroll
         for (int i = 1; i < ITEMS; i++)
-          if (i < cnt && less(mx, k[i])) mx = k[i];
+          if (i < cnt && less(mx, k[i])) { mx = k[i]; vmx = v[i]; }
+        if constexpr (kHasVal<Val>) {
+          int reps = 0;
+#pragma unroll
+          for (int i = 0; i < ITEMS; i++)
+            if (i < cnt && !less(k[i], mx)) reps++;
+          stable_path = reps > 1;
+        }
 #pragma unroll
         for (int i = 0; i < ITEMS; i++) {
           if (i >= cnt) {
             k[i] = mx;
-            if constexpr (kHasVal<Val>) v[i] = v[0];
+            v[i] = vmx;
           }
         }
-        transposition_sort<ITEMS>(k, v, less);
+      }
+      if constexpr (kHasVal<Val>) {
+        if (stable_path) transposition_sort<ITEMS>(k, v, less);
+        else oem_sort<0, ITEMS>(k, v, less);
+      } else {
+        oem_sort<0, ITEMS>(k, v, less);
       }
 #pragma unroll
       for (int i = 0; i < ITEMS; i++) {
@@ -294,49 +358,19 @@ struct CtaSort {
         }
       }
     }
-    __syncthreads();
+    __syncwarp();
+    // Rounds whose merged pairs (2w keys) lie inside one warp's 32*ITEMS keys
+    // only synchronise the warp; wider rounds synchronise the block.
     for (int w = ITEMS; w < m; w *= 2) {
+      const bool blk = NT > 32 && 2 * w > 32 * ITEMS;
+      if (blk) __syncthreads();
       if (cnt > 0) {
         const int ps = (base / (2 * w)) * (2 * w);
-        const int a0 = ps, aLen = min(w, m - ps);
-        const int b0 = ps + w, bLen = max(0, min(w, m - ps - w));
-        const int diag = base - ps;
-        int lo = max(0, diag - bLen), hi = min(diag, aLen);
-        while (lo < hi) {                                  // merge path (stable: A first)
-          int mid = (lo + hi) >> 1;
-          Key a = sk[phys(a0 + mid)], b = sk[phys(b0 + diag - 1 - mid)];
-          if (less(b, a)) hi = mid; else lo = mid + 1;
-        }
-        int ai = lo, bi = diag - lo;
-        const int aLast = a0 + aLen - 1, bLast = b0 + max(bLen - 1, 0);
-        Key ka = sk[phys(min(a0 + ai, aLast))];
-        Key kb = sk[phys(min(b0 + bi, bLast))];
-        Val va, vb;
-        if constexpr (kHasVal<Val>) {
-          va = sv[phys(min(a0 + ai, aLast))];
-          vb = sv[phys(min(b0 + bi, bLast))];
-        }
-#pragma unroll
-        for (int i = 0; i < ITEMS; i++) {
-          bool takeA = (bi >= bLen) || (ai < aLen && !less(kb, ka));
-          k[i] = takeA ? ka : kb;
-          if constexpr (kHasVal<Val>) v[i] = takeA ? va : vb;
-          if (i + 1 < ITEMS) {
-            ai += takeA ? 1 : 0;
-            bi += takeA ? 0 : 1;
-            int idx = takeA ? min(a0 + ai, aLast) : min(b0 + bi, bLast);
-            Key x = sk[phys(idx)];
-            ka = takeA ? x : ka;
-            kb = takeA ? kb : x;
-            if constexpr (kHasVal<Val>) {
-              Val y = sv[phys(idx)];
-              va = takeA ? y : va;
-              vb = takeA ? vb : y;
-            }
-          }
-        }
+        const int aLen = min(w, m - ps);
+        const int bLen = max(0, min(w, m - ps - w));
+        merge_items(sk, sv, ps, aLen, ps + w, bLen, base - ps, k, v, less);
       }
-      __syncthreads();
+      if (blk) __syncthreads(); else __syncwarp();
       if (cnt > 0) {
 #pragma unroll
         for (int i = 0; i < ITEMS; i++) {
@@ -346,8 +380,9 @@ struct CtaSort {
           }
         }
       }
-      __syncthreads();
+      if (!blk) __syncwarp();
     }
+    bar();
   }
 };
 

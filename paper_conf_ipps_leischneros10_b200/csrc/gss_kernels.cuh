@@ -15,9 +15,9 @@
 namespace gss {
 
 constexpr int kClsThreads = 256;
-constexpr int kScatterThreads = 256;
+constexpr int kScatterThreads = 512;
 constexpr int kScatterIter = 8;                                   // keys per thread per chunk
-constexpr int kChunk = kScatterThreads * kScatterIter;            // 2048 keys staged per chunk
+constexpr int kChunk = kScatterThreads * kScatterIter;            // 4096 keys staged per chunk
 constexpr int kScanCtas = 256;
 constexpr int kScanThreads = 256;
 constexpr int kPlanThreads = 256;
@@ -138,35 +138,70 @@ __global__ void k_set_splitters(Ctx<Key, Val, IdT> c) {
 // per-group arrays) in shared memory, then their vector sum
 // (P:320-321).
 // ---------------------------------------------------------------------------
-template <int LOGK, class Key, class IdT, class Cmp>
+// Shared-memory access by 32-bit shared-window address.
+template <class Key>
+__device__ __forceinline__ Key ld_shared(uint32_t a) {
+  if constexpr (sizeof(Key) == 8) {
+    unsigned long long x;
+    asm volatile("ld.shared.u64 %0, [%1];" : "=l"(x) : "r"(a));
+    return (Key)x;
+  } else {
+    uint32_t x;
+    asm volatile("ld.shared.u32 %0, [%1];" : "=r"(x) : "r"(a));
+    return (Key)x;
+  }
+}
+__device__ __forceinline__ void red_shared_add(uint32_t a, uint32_t v) {
+  asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(a), "r"(v));
+}
+
+// U keys per thread in flight; the descent depth log2(k_s) is uniform per
+// tile, so it is a runtime loop around a fully unrolled U-key body.  The
+// tree index j is kept as a shared-memory byte address a = tb + w*j, so each
+// level of Algorithm 2 (j := 2j + (e > bt[j])) is one load, the comparison
+// and a' = 2a - tb + w*[bt[j] < e].
+template <class Key, class IdT, class Cmp>
 __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* __restrict__ ids, uint32_t beg,
-                                              uint32_t len, const Key* tree, const Key* spl, uint32_t ks,
-                                              uint32_t K, bool eq, bool clamp, uint32_t* wc, Cmp less) {
-  constexpr int U = 4;
+                                              uint32_t len, uint32_t tree_s, const Key* spl, uint32_t logk,
+                                              uint32_t ks, uint32_t K, bool eq, bool clamp, uint32_t wc_s, Cmp less) {
+  constexpr int U = 8;
+  constexpr uint32_t W = sizeof(Key);
+  const uint32_t step0 = 0u - tree_s, step1 = W - tree_s;
+  const Key* sp = src + beg;
+  IdT* ip = ids + beg;
   for (uint32_t i0 = threadIdx.x; i0 < len; i0 += U * kClsThreads) {
     Key e[U];
+    uint32_t a[U];
 #pragma unroll
     for (int u = 0; u < U; u++) {
-      uint32_t i = i0 + u * kClsThreads;
-      if (i < len) e[u] = src[beg + i];
+      const uint32_t i = i0 + u * kClsThreads;
+      a[u] = tree_s + W;
+      if (i < len) e[u] = sp[i];
+    }
+    for (uint32_t d = 0; d < logk; d++) {
+#pragma unroll
+      for (int u = 0; u < U; u++) {
+        const Key x = ld_shared<Key>(a[u]);
+        a[u] = a[u] + a[u] + (less(x, e[u]) ? step1 : step0);
+      }
     }
 #pragma unroll
     for (int u = 0; u < U; u++) {
-      uint32_t i = i0 + u * kClsThreads;
+      const uint32_t i = i0 + u * kClsThreads;
       if (i < len) {
-        uint32_t b = descend<LOGK>(tree, e[u], less);
-        uint32_t id;
+        const uint32_t b = (a[u] - tree_s) / W - (1u << logk);
+        uint32_t id = b;
         if (eq) id = 2 * b + ((b + 1 < ks && !less(e[u], spl[b])) ? 1u : 0u);
-        else id = clamp ? min(b, K - 1) : b;
-        ids[beg + i] = (IdT)id;
-        atomicAdd(&wc[id], 1u);
+        else if (clamp) id = min(b, K - 1);
+        ip[i] = (IdT)id;
+        red_shared_add(wc_s + 4 * id, 1u);
       }
     }
   }
 }
 
 template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kClsThreads) k_classify(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+__global__ void __launch_bounds__(kClsThreads, 4) k_classify(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   Key* tree = reinterpret_cast<Key*>(smem_raw);
   Key* spl = tree + kmax;
@@ -191,16 +226,9 @@ __global__ void __launch_bounds__(kClsThreads) k_classify(Ctx<Key, Val, IdT> c, 
     const uint32_t tl = t - B.tile_start;
     const uint32_t beg = B.lo + tl * c.T;
     const uint32_t len = min(c.T, B.m - tl * c.T);
-    uint32_t* wc = wcnt + w * kmax;
-    const bool eq = B.eq != 0, clamp = B.clamp != 0;
-    switch (ilog2(B.ks)) {
-#define GSS_CLS_CASE(L) \
-  case L: classify_tile<L>(src, c.ids, beg, len, tree, spl, B.ks, B.K, eq, clamp, wc, less); break;
-      GSS_CLS_CASE(0) GSS_CLS_CASE(1) GSS_CLS_CASE(2) GSS_CLS_CASE(3) GSS_CLS_CASE(4) GSS_CLS_CASE(5)
-      GSS_CLS_CASE(6) GSS_CLS_CASE(7) GSS_CLS_CASE(8) GSS_CLS_CASE(9) GSS_CLS_CASE(10)
-#undef GSS_CLS_CASE
-      default: break;
-    }
+    const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + w * kmax);
+    const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
+    classify_tile(src, c.ids, beg, len, tree_s, spl, ilog2(B.ks), B.ks, B.K, B.eq != 0, B.clamp != 0, wc_s, less);
     __syncthreads();
     uint32_t* hist = c.hist[slot] + B.hist_base;
     for (uint32_t id = threadIdx.x; id < B.K; id += kClsThreads) {
@@ -273,36 +301,155 @@ __global__ void __launch_bounds__(kScanThreads) k_scan_final(Ctx<Key, Val, IdT> 
 // paper tried, re-adopted for B200) so each bucket's run is
 // written with coalesced stores.
 // ---------------------------------------------------------------------------
-template <class Key, class Val>
+template <class Key, class Val, class IdT>
 struct ScatterSmem {
   static size_t bytes(uint32_t kmax) {
     size_t b = 0;
-    b += (size_t)kmax * 4 * 3;                                  // gbase, ctot, cstart
+    b += (size_t)kmax * 4 * 3;                                  // gbase, ctot, delta
     b += (size_t)(kScatterThreads / 32) * kmax * 4;             // per-warp counters
     b += 64;                                                    // scan scratch
     b = (b + 15) & ~size_t(15);
     b += (size_t)kChunk * sizeof(Key);
     if (kHasVal<Val>) b += (size_t)kChunk * sizeof(Val);
-    b += (size_t)kChunk * 2;                                    // staged ids (u16)
+    b += (size_t)kChunk * sizeof(IdT);                          // staged ids
     return b;
   }
 };
 
+// Predicated shared-memory atomic add (no branch, 32-bit shared address).
+__device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t saddr, uint32_t v) {
+  uint32_t old = 0;
+  asm volatile(
+      "{\n\t.reg .pred p;\n\tsetp.ne.u32 p, %1, 0;\n\t@p atom.shared.add.u32 %0, [%2], %3;\n\t}"
+      : "+r"(old)
+      : "r"(pred), "r"(saddr), "r"(v)
+      : "memory");
+  return old;
+}
+
+// One chunk of <= kChunk keys of a tile: stable rank by (bucket id, position),
+// reorder in shared memory, write each bucket's run with coalesced stores.
+template <bool FULL, class Key, class Val, class IdT>
+__device__ __forceinline__ void scatter_chunk(const Key* __restrict__ ks, const Val* __restrict__ vs,
+                                              const IdT* __restrict__ is, Key* __restrict__ kdst,
+                                              Val* __restrict__ vdst, uint32_t clen, uint32_t K, uint32_t kmax,
+                                              uint32_t* gbase, uint32_t* ctot, uint32_t* delta, uint32_t* wcnt,
+                                              uint32_t* s_warp, Key* skeys, Val* svals, IdT* sids) {
+  constexpr int NW = kScatterThreads / 32;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  const uint32_t ltmask = lanemask_lt();
+  uint32_t* wc = wcnt + w * kmax;
+  for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
+  Key kk[kScatterIter];
+  Val vv[kScatterIter];
+  uint32_t iid[kScatterIter], peers[kScatterIter], old[kScatterIter];
+  const uint32_t q0 = w * (32 * kScatterIter) + lane;
+#pragma unroll
+  for (int it = 0; it < kScatterIter; it++) {
+    const uint32_t q = q0 + it * 32;
+    if (FULL || q < clen) {
+      kk[it] = ks[q];
+      iid[it] = is[q];
+      if constexpr (kHasVal<Val>) vv[it] = vs[q];
+    } else {
+      iid[it] = 0xffffffffu;
+    }
+  }
+  __syncwarp();
+  // peer masks (lanes holding the same bucket id) from one ballot per id bit
+  constexpr int NBITS = sizeof(IdT) == 1 ? 8 : 10;
+#pragma unroll
+  for (int it = 0; it < kScatterIter; it++) {
+    const uint32_t id = iid[it];
+    uint32_t pm = FULL ? kFull : __ballot_sync(kFull, id != 0xffffffffu);
+#pragma unroll
+    for (int bit = 0; bit < NBITS; bit++) {
+      const bool on = (id >> bit) & 1u;
+      const uint32_t bal = __ballot_sync(kFull, on);
+      pm &= on ? bal : ~bal;
+    }
+    peers[it] = pm;
+  }
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
+#pragma unroll
+  for (int it = 0; it < kScatterIter; it++) {
+    // the lowest lane of each group of equal ids adds the group size to the
+    // warp's counter; ranks stay in lane order, hence stable (R7)
+    const uint32_t lead = ((FULL || iid[it] != 0xffffffffu) && (peers[it] & ltmask) == 0) ? 1u : 0u;
+    old[it] = atom_add_shared_if(lead, wc_s + 4 * (iid[it] & 0xffffu), (uint32_t)__popc(peers[it]));
+    __syncwarp();
+  }
+  uint32_t rk[kScatterIter];
+#pragma unroll
+  for (int it = 0; it < kScatterIter; it++)
+    rk[it] = __popc(peers[it] & ltmask) + __shfl_sync(kFull, old[it], __ffs(peers[it]) - 1);
+  __syncthreads();
+  // chunk totals per id, exclusive scan over ids, then every warp's start
+  // within each id folded into its counter (one lookup per key below)
+  const uint32_t per = (K + kScatterThreads - 1) / kScatterThreads;
+  const uint32_t i0 = threadIdx.x * per;
+  uint32_t tsum = 0;
+  for (uint32_t j = 0; j < per; j++) {
+    const uint32_t id = i0 + j;
+    if (id < K) {
+      uint32_t t = 0;
+#pragma unroll
+      for (int q = 0; q < NW; q++) t += wcnt[q * kmax + id];
+      ctot[id] = t;
+      tsum += t;
+    }
+  }
+  uint32_t ex = block_exclusive_scan<kScatterThreads>(tsum, s_warp, nullptr);
+  for (uint32_t j = 0; j < per; j++) {
+    const uint32_t id = i0 + j;
+    if (id < K) {
+      uint32_t run = ex;
+#pragma unroll
+      for (int q = 0; q < NW; q++) {
+        const uint32_t x = wcnt[q * kmax + id];
+        wcnt[q * kmax + id] = run;
+        run += x;
+      }
+      delta[id] = gbase[id] - ex;                         // global = delta + staged position
+      gbase[id] += ctot[id];
+      ex = run;
+    }
+  }
+  __syncthreads();
+#pragma unroll
+  for (int it = 0; it < kScatterIter; it++) {
+    if (FULL || iid[it] != 0xffffffffu) {
+      const uint32_t pos = wc[iid[it]] + rk[it];
+      skeys[pos] = kk[it];
+      if constexpr (kHasVal<Val>) svals[pos] = vv[it];
+      sids[pos] = (IdT)iid[it];
+    }
+  }
+  __syncthreads();
+#pragma unroll 4
+  for (uint32_t q = threadIdx.x; q < (FULL ? (uint32_t)kChunk : clen); q += kScatterThreads) {
+    const uint32_t d = delta[sids[q]] + q;
+    kdst[d] = skeys[q];
+    if constexpr (kHasVal<Val>) vdst[d] = svals[q];
+  }
+  __syncthreads();
+}
+
 template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kScatterThreads) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+__global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   constexpr int NW = kScatterThreads / 32;
   uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);
   uint32_t* ctot = gbase + kmax;
-  uint32_t* cstart = ctot + kmax;
-  uint32_t* wcnt = cstart + kmax;
+  uint32_t* delta = ctot + kmax;
+  uint32_t* wcnt = delta + kmax;
   uint32_t* s_warp = wcnt + NW * kmax;
   size_t off = ((size_t)(kmax * 3 + NW * kmax) * 4 + 64 + 15) & ~size_t(15);
   Key* skeys = reinterpret_cast<Key*>(smem_raw + off);
   off += (size_t)kChunk * sizeof(Key);
   Val* svals = reinterpret_cast<Val*>(smem_raw + off);
   if constexpr (kHasVal<Val>) off += (size_t)kChunk * sizeof(Val);
-  uint16_t* sids = reinterpret_cast<uint16_t*>(smem_raw + off);
+  IdT* sids = reinterpret_cast<IdT*>(smem_raw + off);
 
   const uint32_t slot = level & 1;
   const uint32_t nt = c.cnt->lvl[level].num_tiles;
@@ -312,8 +459,6 @@ __global__ void __launch_bounds__(kScatterThreads) k_scatter(Ctx<Key, Val, IdT> 
   const Val* vsrc = nullptr;
   Val* vdst = nullptr;
   if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
-  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  const uint32_t ltmask = lanemask_lt();
 
   for (uint32_t t = blockIdx.x; t < nt; t += gridDim.x) {
     const uint32_t b = c.tile_bucket[slot][t];
@@ -324,81 +469,18 @@ __global__ void __launch_bounds__(kScatterThreads) k_scatter(Ctx<Key, Val, IdT> 
     const uint32_t* hist = c.hist[slot] + B.hist_base;
     const uint32_t hb = hist[0];
     for (uint32_t id = threadIdx.x; id < B.K; id += kScatterThreads) gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
-    const uint32_t K = B.K;
     for (uint32_t c0 = 0; c0 < len; c0 += kChunk) {
       const uint32_t clen = min((uint32_t)kChunk, len - c0);
-      uint32_t* wc = wcnt + w * kmax;
-      for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
-      __syncwarp();
-      Key kk[kScatterIter];
-      Val vv[kScatterIter];
-      uint32_t iid[kScatterIter], rk[kScatterIter];
-#pragma unroll
-      for (int it = 0; it < kScatterIter; it++) {
-        const uint32_t q = w * (32 * kScatterIter) + it * 32 + lane;
-        iid[it] = 0xffffffffu;
-        if (q < clen) {
-          kk[it] = ksrc[beg + c0 + q];
-          iid[it] = c.ids[beg + c0 + q];
-          if constexpr (kHasVal<Val>) vv[it] = vsrc[beg + c0 + q];
-        }
-      }
-#pragma unroll
-      for (int it = 0; it < kScatterIter; it++) {
-        const uint32_t id = iid[it];
-        const uint32_t peers = __match_any_sync(kFull, id);
-        const uint32_t lt = __popc(peers & ltmask);
-        uint32_t cv = 0;
-        if (id != 0xffffffffu) cv = wc[id];
-        rk[it] = cv + lt;
-        __syncwarp();
-        if (id != 0xffffffffu && lt == 0) wc[id] = cv + __popc(peers);
-        __syncwarp();
-      }
-      __syncthreads();
-      for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) {
-        uint32_t run = 0;
-#pragma unroll
-        for (int q = 0; q < NW; q++) {
-          uint32_t x = wcnt[q * kmax + id];
-          wcnt[q * kmax + id] = run;
-          run += x;
-        }
-        ctot[id] = run;
-      }
-      __syncthreads();
-      {
-        // exclusive scan of ctot over ids -> cstart (each thread owns a run of ids)
-        const uint32_t per = (K + kScatterThreads - 1) / kScatterThreads;
-        const uint32_t i0 = threadIdx.x * per;
-        uint32_t s = 0;
-        for (uint32_t j = 0; j < per; j++)
-          if (i0 + j < K) s += ctot[i0 + j];
-        uint32_t ex = block_exclusive_scan<kScatterThreads>(s, s_warp, nullptr);
-        for (uint32_t j = 0; j < per; j++)
-          if (i0 + j < K) { cstart[i0 + j] = ex; ex += ctot[i0 + j]; }
-      }
-      __syncthreads();
-#pragma unroll
-      for (int it = 0; it < kScatterIter; it++) {
-        const uint32_t id = iid[it];
-        if (id != 0xffffffffu) {
-          const uint32_t pos = cstart[id] + wc[id] + rk[it];
-          skeys[pos] = kk[it];
-          if constexpr (kHasVal<Val>) svals[pos] = vv[it];
-          sids[pos] = (uint16_t)id;
-        }
-      }
-      __syncthreads();
-      for (uint32_t q = threadIdx.x; q < clen; q += kScatterThreads) {
-        const uint32_t id = sids[q];
-        const uint32_t d = gbase[id] + (q - cstart[id]);
-        kdst[d] = skeys[q];
-        if constexpr (kHasVal<Val>) vdst[d] = svals[q];
-      }
-      __syncthreads();
-      for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] += ctot[id];
-      __syncthreads();
+      const Key* ks = ksrc + beg + c0;
+      const Val* vs = nullptr;
+      if constexpr (kHasVal<Val>) vs = vsrc + beg + c0;
+      const IdT* is = c.ids + beg + c0;
+      if (clen == (uint32_t)kChunk)
+        scatter_chunk<true>(ks, vs, is, kdst, vdst, clen, B.K, kmax, gbase, ctot, delta, wcnt, s_warp, skeys, svals,
+                            sids);
+      else
+        scatter_chunk<false>(ks, vs, is, kdst, vdst, clen, B.K, kmax, gbase, ctot, delta, wcnt, s_warp, skeys, svals,
+                             sids);
     }
   }
 }
@@ -409,15 +491,33 @@ __global__ void __launch_bounds__(kScatterThreads) k_scatter(Ctx<Key, Val, IdT> 
 // (m > M), an in-SM sort item (m <= M), a final equality bucket (R4), or --
 // past the last launched level -- an overflow item.
 // ---------------------------------------------------------------------------
-template <class Key, class Val, class IdT>
-__device__ __forceinline__ void push_small(const Ctx<Key, Val, IdT>& c, uint32_t lo, uint32_t m, uint32_t buf) {
-  uint32_t cls = 0;
-  while (cls + 1 < kNumClasses && m > c.class_cap[cls]) cls++;
-  uint32_t i = atomicAdd(&c.cnt->small_count[cls], 1u);
-  if (i < c.cap_small[cls]) c.small[cls][i] = Item{lo, m, buf, 0};
-  else atomicOr(&c.cnt->err, 1u);
-  atomicAdd(&c.cnt->small_elems, (unsigned long long)m);
-  atomicMax(&c.cnt->max_small, (unsigned long long)m);
+// Warp-aggregated append of `cnt` items per lane to a list with counter
+// *ctr: returns each lane's first slot (lanes with cnt == 0 get garbage).
+// All 32 lanes must call it.
+__device__ __forceinline__ uint32_t warp_append(uint32_t* ctr, uint32_t cnt) {
+  const int lane = threadIdx.x & 31;
+  uint32_t incl = cnt;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    uint32_t y = __shfl_up_sync(kFull, incl, o);
+    if (lane >= o) incl += y;
+  }
+  const uint32_t total = __shfl_sync(kFull, incl, 31);
+  uint32_t base = 0;
+  if (lane == 0 && total) base = atomicAdd(ctr, total);
+  base = __shfl_sync(kFull, base, 0);
+  return base + incl - cnt;
+}
+
+__device__ __forceinline__ uint64_t warp_sum64(uint64_t x) {
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(kFull, x, o);
+  return x;
+}
+__device__ __forceinline__ uint32_t warp_max32(uint32_t x) {
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) x = max(x, __shfl_xor_sync(kFull, x, o));
+  return x;
 }
 
 template <class Key, class Val, class IdT>
@@ -426,56 +526,95 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
   const uint32_t nb = c.cnt->lvl[level].num_buckets;
   const uint32_t db = c.dst(level);
   const uint32_t next = level + 1;
+  const int lane = threadIdx.x & 31;
+  const uint32_t cap_last = c.class_cap[kNumClasses - 1];
   for (uint32_t b = blockIdx.x; b < nb; b += gridDim.x) {
     const Bucket B = c.bk[slot][b];
     const uint32_t* hist = c.hist[slot] + B.hist_base;
     const uint32_t hb = hist[0];
-    for (uint32_t id = threadIdx.x; id < B.K; id += kPlanThreads) {
-      const uint32_t start = hist[id * B.ntiles] - hb + B.lo;
-      const uint32_t end = (id + 1 < B.K) ? hist[(id + 1) * B.ntiles] - hb + B.lo : B.lo + B.m;
-      const uint32_t m = end - start;
-      if (m == 0) continue;
-      const bool is_eq = B.eq && (id & 1);
-      if (is_eq) {
-        atomicAdd(&c.cnt->eq_buckets, 1ull);
-        atomicAdd(&c.cnt->eq_elems, (unsigned long long)m);
-        if (db == BUF_OUT) continue;                       // all keys equal and already in place
-        if (m <= c.class_cap[kNumClasses - 1]) {
-          push_small(c, start, m, db);
-        } else {
-          uint32_t nt = (m + c.T - 1) / c.T;
-          uint32_t i = atomicAdd(&c.cnt->copy_count, nt);
+    for (uint32_t id0 = 0; id0 < B.K; id0 += kPlanThreads) {         // uniform trip count
+      const uint32_t id = id0 + threadIdx.x;
+      uint32_t start = 0, m = 0;
+      if (id < B.K) {
+        start = hist[id * B.ntiles] - hb + B.lo;
+        const uint32_t end = (id + 1 < B.K) ? hist[(id + 1) * B.ntiles] - hb + B.lo : B.lo + B.m;
+        m = end - start;
+      }
+      const bool is_eq = m && B.eq && (id & 1);
+      // categories: small-sort class, copy (big equality bucket), next level, overflow
+      const bool to_small = m && ((is_eq && db != BUF_OUT && m <= cap_last) || (!is_eq && m <= c.M));
+      const bool to_copy = is_eq && db != BUF_OUT && m > cap_last;
+      const bool to_next = m && !is_eq && m > c.M && next < c.L;
+      const bool to_ovf = m && !is_eq && m > c.M && next >= c.L;
+      // equality-bucket statistics
+      {
+        const uint64_t e_cnt = warp_sum64(is_eq ? 1 : 0), e_el = warp_sum64(is_eq ? m : 0);
+        if (lane == 0 && e_cnt) {
+          atomicAdd(&c.cnt->eq_buckets, (unsigned long long)e_cnt);
+          atomicAdd(&c.cnt->eq_elems, (unsigned long long)e_el);
+        }
+      }
+      // in-SM sort lists, one per size class
+      uint32_t cls = 0;
+      while (cls + 1 < kNumClasses && m > c.class_cap[cls]) cls++;
+      for (int q = 0; q < kNumClasses; q++) {
+        const bool mine = to_small && cls == (uint32_t)q;
+        if (!__any_sync(kFull, mine)) continue;
+        const uint32_t i = warp_append(&c.cnt->small_count[q], mine ? 1u : 0u);
+        if (mine) {
+          if (i < c.cap_small[q]) c.small[q][i] = Item{start, m, db, 0};
+          else atomicOr(&c.cnt->err, 1u);
+        }
+      }
+      {
+        const uint64_t s_el = warp_sum64(to_small ? m : 0);
+        const uint32_t s_max = warp_max32(to_small ? m : 0);
+        if (lane == 0 && s_el) {
+          atomicAdd(&c.cnt->small_elems, (unsigned long long)s_el);
+          atomicMax(&c.cnt->max_small, (unsigned long long)s_max);
+        }
+      }
+      if (__any_sync(kFull, to_copy)) {
+        const uint32_t nt = to_copy ? (m + c.T - 1) / c.T : 0;
+        const uint32_t i = warp_append(&c.cnt->copy_count, nt);
+        if (to_copy) {
           if (i + nt <= c.cap_copy) {
             for (uint32_t q = 0; q < nt; q++) c.copy[i + q] = Item{start + q * c.T, min(c.T, m - q * c.T), db, 0};
           } else {
             atomicOr(&c.cnt->err, 2u);
           }
         }
-      } else if (m <= c.M) {
-        push_small(c, start, m, db);
-      } else if (next < c.L) {
-        const uint32_t kb = choose_kb(c.k, c.k_policy, c.fill_div, c.M, m);
-        const uint32_t nt = (m + c.T - 1) / c.T;
+      }
+      if (__any_sync(kFull, to_next)) {
         LevelCounters& NL = c.cnt->lvl[next];
-        const uint32_t bi = atomicAdd(&NL.num_buckets, 1u);
-        const uint32_t ts = atomicAdd(&NL.num_tiles, nt);
-        const uint32_t hbn = atomicAdd(&NL.hist_alloc, max(kb, 3u) * nt);
-        const uint32_t sbn = atomicAdd(&NL.spl_alloc, 2 * kb);
-        atomicAdd(&NL.split_elems, (unsigned long long)m);
-        if (bi < c.cap_buckets && ts + nt <= c.cap_tiles && hbn + max(kb, 3u) * nt <= c.cap_hist &&
-            sbn + 2 * kb <= c.cap_spl) {
-          Bucket nbk{};
-          nbk.lo = start; nbk.m = m; nbk.tile_start = ts; nbk.ntiles = nt; nbk.kb = kb;
-          nbk.hist_base = hbn; nbk.spl_base = sbn;
-          c.bk[next & 1][bi] = nbk;
-        } else {
-          atomicOr(&c.cnt->err, 4u);
+        const uint32_t kb = to_next ? choose_kb(c.k, c.k_policy, c.fill_div, c.M, m) : 0;
+        const uint32_t nt = to_next ? (m + c.T - 1) / c.T : 0;
+        const uint32_t bi = warp_append(&NL.num_buckets, to_next ? 1u : 0u);
+        const uint32_t ts = warp_append(&NL.num_tiles, nt);
+        const uint32_t hbn = warp_append(&NL.hist_alloc, to_next ? max(kb, 3u) * nt : 0u);
+        const uint32_t sbn = warp_append(&NL.spl_alloc, 2 * kb);
+        const uint64_t el = warp_sum64(to_next ? m : 0);
+        if (lane == 0 && el) atomicAdd(&NL.split_elems, (unsigned long long)el);
+        if (to_next) {
+          if (bi < c.cap_buckets && ts + nt <= c.cap_tiles && hbn + max(kb, 3u) * nt <= c.cap_hist &&
+              sbn + 2 * kb <= c.cap_spl) {
+            Bucket nbk{};
+            nbk.lo = start; nbk.m = m; nbk.tile_start = ts; nbk.ntiles = nt; nbk.kb = kb;
+            nbk.hist_base = hbn; nbk.spl_base = sbn;
+            c.bk[next & 1][bi] = nbk;
+          } else {
+            atomicOr(&c.cnt->err, 4u);
+          }
         }
-      } else {
-        uint32_t i = atomicAdd(&c.cnt->ovf_count, 1u);
-        if (i < c.cap_ovf) c.ovf[i] = Item{start, m, db, 0};
-        else atomicOr(&c.cnt->err, 8u);
-        atomicAdd(&c.cnt->ovf_elems, (unsigned long long)m);
+      }
+      if (__any_sync(kFull, to_ovf)) {
+        const uint32_t i = warp_append(&c.cnt->ovf_count, to_ovf ? 1u : 0u);
+        const uint64_t el = warp_sum64(to_ovf ? m : 0);
+        if (lane == 0 && el) atomicAdd(&c.cnt->ovf_elems, (unsigned long long)el);
+        if (to_ovf) {
+          if (i < c.cap_ovf) c.ovf[i] = Item{start, m, db, 0};
+          else atomicOr(&c.cnt->err, 8u);
+        }
       }
     }
   }
@@ -485,16 +624,21 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
 // Sorting buckets: one CTA per bucket of at most M keys; the
 // bucket is loaded to shared memory, sorted by CtaSort, written to keys_out.
 // ---------------------------------------------------------------------------
-template <class Key, class Val, class IdT, class Cmp, int NT>
-__global__ void __launch_bounds__(NT, 1) k_small(Ctx<Key, Val, IdT> c, uint32_t cls) {
+template <class Key, class Val, int CAP>
+constexpr int small_threads() { return CAP / sort_items<Key, Val>(); }
+
+template <class Key, class Val, class IdT, class Cmp, int CAP, int NT = small_threads<Key, Val, CAP>()>
+__global__ void __launch_bounds__(NT, (1024 / NT) > 0 ? 1024 / NT : 1)
+    k_small(Ctx<Key, Val, IdT> c, uint32_t cls, uint32_t retry) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   using Sorter = CtaSort<Key, Val, NT, Cmp>;
   Key* sk = reinterpret_cast<Key*>(smem_raw);
   Val* sv = reinterpret_cast<Val*>(smem_raw + (size_t)Sorter::PL * sizeof(Key));
   const Cmp less;
-  const uint32_t ni = min(c.cnt->small_count[cls], c.cap_small[cls]);
+  const uint32_t ni = min(retry ? c.cnt->retry_count[cls] : c.cnt->small_count[cls], c.cap_small[cls]);
+  const Item* list = retry ? c.retry[cls] : c.small[cls];
   for (uint32_t i = blockIdx.x; i < ni; i += gridDim.x) {
-    const Item I = c.small[cls][i];
+    const Item I = list[i];
     const Key* src = c.keys(I.buf);
     for (uint32_t q = threadIdx.x; q < I.m; q += NT) sk[phys(q)] = src[I.lo + q];
     if constexpr (kHasVal<Val>) {
@@ -505,6 +649,236 @@ __global__ void __launch_bounds__(NT, 1) k_small(Ctx<Key, Val, IdT> c, uint32_t 
     for (uint32_t q = threadIdx.x; q < I.m; q += NT) c.kout[I.lo + q] = sk[phys(q)];
     if constexpr (kHasVal<Val>)
       for (uint32_t q = threadIdx.x; q < I.m; q += NT) c.vout[I.lo + q] = sv[phys(q)];
+    __syncthreads();
+  }
+}
+
+// ---------------------------------------------------------------------------
+// In-SM bucket sort by one more sample-sort split inside shared memory
+// (the paper's "sample sort based" chunk sorter, re-derived for
+// B200): a warp sorts a sample of 4*k2 keys and takes k2-1 splitters; the
+// CTA classifies the bucket (Algorithm 2 descent in shared memory), counts,
+// and places every key into its sub-bucket's region of shared memory; then
+// each warp merge-sorts whole sub-buckets (odd-even merge network + merge
+// path) with warp barriers only and writes them to keys_out.
+// Equality sub-buckets (R4) need no sorting.  A sub-bucket larger than one
+// warp's capacity is written unsorted and retried by k_small.
+// ---------------------------------------------------------------------------
+constexpr int kSplitMaxK = 128;            // k2 <= 128 sub-buckets (K <= 255 ids)
+constexpr int kSplitPad = 256;             // per-region padding slack (one per id)
+
+template <class Key, class Val, int CAP, int NT>
+struct SplitSortSmem {
+  static constexpr int NW = NT / 32;
+  static constexpr int PL = padded_len(CAP) + kSplitPad + 16;
+  __host__ __device__ static constexpr size_t off_vals() { return (size_t)PL * sizeof(Key); }
+  __host__ __device__ static constexpr size_t off_ids() { return off_vals() + (kHasVal<Val> ? (size_t)PL * sizeof(Val) : 0); }
+  __host__ __device__ static constexpr size_t off_tree() { return (off_ids() + CAP + 15) & ~size_t(15); }
+  __host__ __device__ static constexpr size_t off_spl() { return off_tree() + kSplitMaxK * sizeof(Key); }
+  __host__ __device__ static constexpr size_t off_wcnt() { return off_spl() + kSplitMaxK * sizeof(Key); }
+  __host__ __device__ static constexpr size_t off_tot() { return off_wcnt() + (size_t)NW * 256 * 4; }
+  __host__ __device__ static constexpr size_t off_cst() { return off_tot() + 256 * 4; }
+  __host__ __device__ static constexpr size_t off_rst() { return off_cst() + 256 * 4; }
+  __host__ __device__ static constexpr size_t off_misc() { return off_rst() + 256 * 4; }
+  __host__ __device__ static constexpr size_t bytes() { return off_misc() + 16 * 4; }
+};
+
+template <class Key, class Val, int CAP>
+constexpr int split_threads() { return 256; }
+
+// Warp-level sorts called out of line (keeps the split kernel's registers low).
+template <class Key, class Val, class Cmp, int ITEMS>
+__device__ __forceinline__ void warp_sort(Key* rk, Val* rv, int t) {
+  CtaSort<Key, Val, 32, Cmp, ITEMS>::sort(rk, rv, t, Cmp());
+}
+
+template <class Key, class Val, class IdT, class Cmp, int CAP, int NT = split_threads<Key, Val, CAP>()>
+__global__ void __launch_bounds__(NT, 2) k_split_sort(Ctx<Key, Val, IdT> c, uint32_t cls) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  using L = SplitSortSmem<Key, Val, CAP, NT>;
+  using WSort = CtaSort<Key, Val, 32, Cmp>;                 // one warp: 32*ITEMS keys
+  using WSort4 = CtaSort<Key, Val, 32, Cmp, 4>;             // smaller sub-buckets: all lanes busy
+  using WSort8 = CtaSort<Key, Val, 32, Cmp, 8>;
+  constexpr int NW = NT / 32;
+  constexpr int WCAP = WSort::C;
+  Key* sk = reinterpret_cast<Key*>(smem_raw);
+  Val* sv = reinterpret_cast<Val*>(smem_raw + L::off_vals());
+  uint8_t* sid = smem_raw + L::off_ids();
+  Key* tree = reinterpret_cast<Key*>(smem_raw + L::off_tree());
+  Key* spl = reinterpret_cast<Key*>(smem_raw + L::off_spl());
+  uint32_t* wcnt = reinterpret_cast<uint32_t*>(smem_raw + L::off_wcnt());
+  uint32_t* tot = reinterpret_cast<uint32_t*>(smem_raw + L::off_tot());
+  uint32_t* cst = reinterpret_cast<uint32_t*>(smem_raw + L::off_cst());
+  uint32_t* rst = reinterpret_cast<uint32_t*>(smem_raw + L::off_rst());
+  uint32_t* misc = reinterpret_cast<uint32_t*>(smem_raw + L::off_misc());
+  const Cmp less;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + w * 256);
+  const uint32_t ni = min(c.cnt->small_count[cls], c.cap_small[cls]);
+  for (uint32_t it = blockIdx.x; it < ni; it += gridDim.x) {
+    const Item I = c.small[cls][it];
+    const uint32_t m = I.m;
+    const Key* src = c.keys(I.buf) + I.lo;
+    const Val* vsrc = nullptr;
+    if constexpr (kHasVal<Val>) vsrc = c.vals(I.buf) + I.lo;
+    Key* kout = c.kout + I.lo;
+    Val* vout = nullptr;
+    if constexpr (kHasVal<Val>) vout = c.vout + I.lo;
+    // ---- 1. sample and splitters (warp 0); the other warps clear counters
+    uint32_t k2 = 2;                                   // sub-buckets of about WCAP/4 keys
+    while (k2 < kSplitMaxK && k2 * (WCAP / 4) < m) k2 <<= 1;
+    const uint32_t s = 4 * k2;
+    for (uint32_t j = threadIdx.x; j < (uint32_t)NW * 256; j += NT) wcnt[j] = 0;
+    if (w == 0) {
+      for (uint32_t j = lane; j < s; j += 32) sk[phys(j)] = src[sample_pos(c.seed, 254, I.lo, j, m)];
+      if (s <= 128) warp_sort<Key, NoVal, Cmp, 4>(sk, nullptr, (int)s);
+      else if (s <= 256) warp_sort<Key, NoVal, Cmp, 8>(sk, nullptr, (int)s);
+      else warp_sort<Key, NoVal, Cmp, 16>(sk, nullptr, (int)s);
+      bool dup = false;
+      for (uint32_t i = lane; i + 2 < k2; i += 32) dup |= !less(sk[phys(4 * (i + 1) - 1)], sk[phys(4 * (i + 2) - 1)]);
+      const bool eq = __any_sync(kFull, dup) || k2 == 2;
+      const uint32_t ks = eq ? max(2u, k2 / 2) : k2;
+      const uint32_t stride = s / ks;
+      for (uint32_t i = lane; i + 1 < ks; i += 32) spl[i] = sk[phys(stride * (i + 1) - 1)];
+      for (uint32_t j = lane + 1; j < ks; j += 32) {
+        const uint32_t d = ilog2(j), q = j - (1u << d);
+        tree[j] = sk[phys(stride * (((2 * q + 1) * ks) >> (d + 1)) - 1)];
+      }
+      if (lane == 0) { misc[0] = ks; misc[1] = eq ? 1u : 0u; misc[2] = eq ? 2 * ks - 1 : ks; misc[3] = 0; }
+    }
+    __syncthreads();
+    const uint32_t ks = misc[0], K = misc[2];
+    const bool eq = misc[1] != 0;
+    const uint32_t logk = ilog2(ks);
+    // ---- 2. classify every key, count per warp (striped: q = r*NT + tid)
+    {
+      constexpr uint32_t W = sizeof(Key);
+      constexpr int U = 8;
+      const uint32_t step0 = 0u - tree_s, step1 = W - tree_s;
+      for (uint32_t q0 = threadIdx.x; q0 < m; q0 += U * NT) {
+        Key e[U];
+        uint32_t a[U];
+#pragma unroll
+        for (int u = 0; u < U; u++) {
+          a[u] = tree_s + W;
+          if (q0 + u * NT < m) e[u] = src[q0 + u * NT];
+        }
+        for (uint32_t d = 0; d < logk; d++) {
+#pragma unroll
+          for (int u = 0; u < U; u++) a[u] = a[u] + a[u] + (less(ld_shared<Key>(a[u]), e[u]) ? step1 : step0);
+        }
+#pragma unroll
+        for (int u = 0; u < U; u++) {
+          const uint32_t q = q0 + u * NT;
+          if (q < m) {
+            uint32_t id = (a[u] - tree_s) / W - ks;
+            if (eq) id = 2 * id + ((id + 1 < ks && !less(e[u], spl[id])) ? 1u : 0u);
+            sid[q] = (uint8_t)id;
+            red_shared_add(wc_s + 4 * id, 1u);
+          }
+        }
+      }
+    }
+    __syncthreads();
+    // ---- 3. sub-bucket sizes, output offsets, padded shared regions, warp cursors
+    if (threadIdx.x < K) {
+      uint32_t t = 0;
+#pragma unroll 4
+      for (int q = 0; q < NW; q++) t += wcnt[q * 256 + threadIdx.x];
+      tot[threadIdx.x] = t;
+    }
+    __syncthreads();
+    if (w == 0) {
+      // K <= 255: one warp scans sizes and padded region sizes
+      uint32_t run_c = 0, run_r = 0;
+      for (uint32_t j0 = 0; j0 < K; j0 += 32) {
+        const uint32_t j = j0 + lane;
+        const uint32_t t = j < K ? tot[j] : 0u;
+        const uint32_t pr = t ? (uint32_t)padded_len((int)t) : 0u;
+        uint32_t ic = t, ir = pr;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+          const uint32_t yc = __shfl_up_sync(kFull, ic, o), yr = __shfl_up_sync(kFull, ir, o);
+          if (lane >= o) { ic += yc; ir += yr; }
+        }
+        if (j < K) { cst[j] = run_c + ic - t; rst[j] = run_r + ir - pr; }
+        run_c += __shfl_sync(kFull, ic, 31);
+        run_r += __shfl_sync(kFull, ir, 31);
+      }
+    }
+    __syncthreads();
+    if (threadIdx.x < K) {
+      const uint32_t j = threadIdx.x;
+      uint32_t run = 0;
+      for (int q = 0; q < NW; q++) {
+        const uint32_t x = wcnt[q * 256 + j];
+        wcnt[q * 256 + j] = run;
+        run += x;
+      }
+    }
+    __syncthreads();
+    // ---- 4. place every key in its sub-bucket region (same striping as step 2)
+    {
+      constexpr int U = 8;
+      for (uint32_t q0 = threadIdx.x; q0 < m; q0 += U * NT) {
+        Key e[U];
+        Val v[U];
+#pragma unroll
+        for (int u = 0; u < U; u++) {
+          const uint32_t q = q0 + u * NT;
+          if (q < m) {
+            e[u] = src[q];
+            if constexpr (kHasVal<Val>) v[u] = vsrc[q];
+          }
+        }
+#pragma unroll
+        for (int u = 0; u < U; u++) {
+          const uint32_t q = q0 + u * NT;
+          if (q < m) {
+            const uint32_t id = sid[q];
+            uint32_t r;
+            asm volatile("atom.shared.add.u32 %0, [%1], 1;" : "=r"(r) : "r"(wc_s + 4 * id));
+            const uint32_t pos = rst[id] + (uint32_t)phys((int)r);
+            sk[pos] = e[u];
+            if constexpr (kHasVal<Val>) sv[pos] = v[u];
+          }
+        }
+      }
+    }
+    __syncthreads();
+    // ---- 5. warps take whole sub-buckets: sort and write out
+    for (;;) {
+      uint32_t j = 0;
+      if (lane == 0) j = atomicAdd(&misc[3], 1u);
+      j = __shfl_sync(kFull, j, 0);
+      if (j >= K) break;
+      const uint32_t t = tot[j];
+      if (t == 0) continue;
+      Key* rk = sk + rst[j];
+      Val* rv = nullptr;
+      if constexpr (kHasVal<Val>) rv = sv + rst[j];
+      const bool needs_sort = t > 1 && !(eq && (j & 1));
+      if (needs_sort && t > (uint32_t)WCAP) {
+        // too large for one warp: write unsorted, retry with the block merge sort
+        if (lane == 0) {
+          uint32_t rc = 0;
+          while (rc + 1 < kNumClasses && t > c.class_cap[rc]) rc++;
+          const uint32_t slot = atomicAdd(&c.cnt->retry_count[rc], 1u);
+          if (slot < c.cap_small[rc]) c.retry[rc][slot] = Item{I.lo + cst[j], t, BUF_OUT, 0};
+          else atomicOr(&c.cnt->err, 16u);
+        }
+      } else if (needs_sort) {
+        if (t <= (uint32_t)WSort4::C && WSort4::C < WCAP) warp_sort<Key, Val, Cmp, 4>(rk, rv, (int)t);
+        else if (t <= (uint32_t)WSort8::C && WSort8::C < WCAP) warp_sort<Key, Val, Cmp, 8>(rk, rv, (int)t);
+        else warp_sort<Key, Val, Cmp, WSort::ITEMS>(rk, rv, (int)t);
+      }
+      for (uint32_t r = lane; r < t; r += 32) {
+        kout[cst[j] + r] = rk[phys((int)r)];
+        if constexpr (kHasVal<Val>) vout[cst[j] + r] = rv[phys((int)r)];
+      }
+      __syncwarp();
+    }
     __syncthreads();
   }
 }

@@ -212,3 +212,17 @@ def test_full_size(gss, oracle_mod, width, n, dist):
     assert mix(x) == mix(y)
     for r in (0, n // 3, n - 1):
         assert int(y[r]) == oracle_mod.select(x, r)
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist", ["uniform", "dd", "and3", "equal"])
+def test_split_sort_variant(gss, width, pairs, dist):
+    """The in-SM sample-split bucket sorter (GSS_FLAG_SPLIT_SORT) gives the same keys."""
+    n = (1 << 19) + 77
+    x = inputs.keys(dist, n, width, seed=2)
+    v = inputs.values(n, width) if pairs else None
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=2, stats=True)
+    assert st.error_flags == 0
+    np.testing.assert_array_equal(to_host(ko), np.sort(x))
+    if pairs:
+        check_pairs(x, to_host(vo), np.sort(x))
