@@ -41,7 +41,8 @@ WORKLOADS = {
     "c1_u32_2p16": (1 << 16, 32, False, "uniform", "2^16 uniform u32 keys, k=128 (BASELINE configs[0]; launch-bound)"),
 }
 DEFAULT_WORKLOAD = "c4_u64_2p28"
-CPU_SAMPLE_N = 1 << 26
+CPU_SAMPLE_N = 1 << 26          # cpu_baseline leg: one oracle sort, ~10 s on one host core
+REF_STEP_N = 1 << 24            # --impl reference: per-step sample, ~2.5 s per step
 
 
 def peaks():
@@ -144,7 +145,7 @@ def run_reference(args, wl):
     import oracle
     oracle.build()
     n, bits, pairs, dist, desc = WORKLOADS[wl]
-    ns = min(n, CPU_SAMPLE_N)
+    ns = min(n, REF_STEP_N)
     x = inputs.keys(dist, ns, bits, seed=1) if dist != "sorted" else inputs.keys(dist, ns, bits)
     v = inputs.values(ns, bits) if pairs else None
     prm = oracle.Params(k=256, a=30, M=8192 if (pairs and bits == 64) else 16384, k_policy=1, fill_div=4, seed=5489)
@@ -207,7 +208,12 @@ def run_ours(args, wl):
     dvals = torch.from_numpy(hv).to(dev) if pairs else None
     stream = torch.cuda.current_stream(dev)
 
-    if world > 1:
+    use_dist = world > 1 or args.force_dist
+    if use_dist:
+        if world == 1 and not dist_mod.is_initialized():
+            os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+            os.environ.setdefault("MASTER_PORT", "29533")
+            dist_mod.init_process_group("nccl", rank=0, world_size=1, device_id=dev)
         from paper_conf_ipps_leischneros10_b200 import dist as gdist
         sorter = gdist.DistSorter(kind, n, pairs, device=dev, **params)
         step = lambda: sorter(dkeys, dvals)  # noqa: E731
@@ -243,7 +249,7 @@ def run_ours(args, wl):
     value = n * world / (ms * 1e-3) / 1e9
 
     # ---- result check (not timed) ----
-    if world == 1:
+    if not use_dist:
         ok = mix_check(x, kout.cpu().numpy())
     else:
         ok = sorter.verify(x)
@@ -253,7 +259,11 @@ def run_ours(args, wl):
     roof = None
     gpu_launches = None
     hbm, peak_src = peaks()
-    if world == 1:
+    if use_dist:
+        gpu_launches = sorter.count_launches(dkeys, dvals) * args.steps
+        extra["exchange"] = {"send_counts": sorter.last_counts[0], "recv_counts": sorter.last_counts[1],
+                             "samples_per_rank": sorter.S}
+    if not use_dist:
         st = sorter(dkeys, kout, dvals, vout, stats=True)
         gpu_launches = st.launches * args.steps
         prof = gss.Profiler()
@@ -284,7 +294,7 @@ def run_ours(args, wl):
                                         "small_buckets": st.small_buckets}
     # ---- end to end through the C ABI with host buffers ----
     e2e = None
-    if world == 1:
+    if not use_dist:
         hs = gss.HostSorter(kind, n, pairs, device=dev, **params)
         hk = torch.from_numpy(x).pin_memory()
         ho = torch.empty_like(hk).pin_memory()
@@ -306,7 +316,7 @@ def run_ours(args, wl):
 
     # ---- CPU baseline: the oracle on a bounded sample (rank 0, N == 1 only) ----
     cpu = None
-    if world == 1 and not args.no_cpu_baseline:
+    if world == 1 and not use_dist and not args.no_cpu_baseline:
         import oracle
         oracle.build()
         ns = min(n, CPU_SAMPLE_N)
@@ -334,7 +344,7 @@ def run_ours(args, wl):
             "clocks": clk.summary(), "result_check": bool(ok), **extra,
         }
         print(json.dumps(line), flush=True)
-    if world > 1:
+    if dist_mod.is_initialized():
         dist_mod.destroy_process_group()
     return 0 if ok else 1
 
@@ -347,6 +357,7 @@ def main():
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--workload", default=DEFAULT_WORKLOAD, choices=sorted(WORKLOADS))
     ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--force-dist", action="store_true", help="use the distributed path even on one GPU")
     args = ap.parse_args()
     if args.warmup < 3 and args.impl == "ours":
         args.warmup = 3

@@ -226,3 +226,29 @@ def test_split_sort_variant(gss, width, pairs, dist):
     np.testing.assert_array_equal(to_host(ko), np.sort(x))
     if pairs:
         check_pairs(x, to_host(vo), np.sort(x))
+
+
+def test_distributed_sorter_single_rank_nccl(gss):
+    """The distributed path on one rank over NCCL: sample, sort, partition_by, all-to-all-v, sort."""
+    import torch.distributed as dist
+    from paper_conf_ipps_leischneros10_b200.dist import DistSorter
+    import os
+    os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+    os.environ.setdefault("MASTER_PORT", "29561")
+    own = not dist.is_initialized()
+    if own:
+        dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
+    try:
+        n = 1 << 20
+        x = inputs.keys("gaussian", n, 64, seed=9)
+        v = inputs.values(n, 64)
+        ds = DistSorter("u64", n, True, device="cuda")
+        k, vv, nr = ds(to_dev(x), to_dev(v))
+        assert nr == n
+        np.testing.assert_array_equal(to_host(k), np.sort(x))
+        check_pairs(x, to_host(vv), np.sort(x))
+        assert ds.verify(x)
+        assert ds.count_launches(to_dev(x), to_dev(v)) > 10
+    finally:
+        if own:
+            dist.destroy_process_group()
