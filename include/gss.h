@@ -103,6 +103,10 @@ typedef struct gss_params {
 
 #define GSS_FLAG_RECOMPUTE_IDS 1u  /* Phase 4 re-descends the tree instead of reading stored
                                       bucket ids (the paper's choice); reserved  */
+#define GSS_FLAG_STABLE 4u         /* Phase 4 ranks keys stably (R7: each level is a stable
+                                      partition); default: one shared atomic per key, which
+                                      partitions correctly but orders keys within a bucket in
+                                      the hardware's atomic order                             */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets with one more sample-sort split inside
                                       shared memory + warp merge sorts (P:332-335 variant)  */
 

@@ -31,7 +31,7 @@ struct gss_profiler {
 namespace {
 
 constexpr uint32_t kVersion = 1;
-constexpr uint32_t kClassCap[kNumClasses] = {2048, 4096, 8192, 16384};
+constexpr uint32_t kClassCap[kNumClasses] = {512, 1024, 2048, 4096, 8192, 16384};
 
 size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -84,7 +84,7 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   const uint32_t cap = max_small_capacity<Key, Val>();
   c->M = p.small_threshold ? p.small_threshold : cap;
   if (c->M > cap) return GSS_ERROR_INVALID_VALUE;
-  c->T = p.tile ? p.tile : 16384;
+  c->T = p.tile ? p.tile : 32768;
   if (c->T < 2048 || c->T % 2048 || c->T > (1u << 24)) return GSS_ERROR_INVALID_VALUE;
   c->k_policy = p.k_policy ? p.k_policy : 1;
   if (c->k_policy > 2) return GSS_ERROR_INVALID_VALUE;
@@ -258,6 +258,7 @@ struct Engine {
     c.sample_cap = 16384;
     c.L = mode == MODE_SORT ? cfg.L : 1;
     c.mode = mode;
+    c.stable = ((cfg.flags & GSS_FLAG_STABLE) || mode != MODE_SORT) ? 1u : 0u;   // partitions stay stable (R7 probe)
     c.cap_buckets = lay.cap_buckets; c.cap_tiles = lay.cap_tiles; c.cap_hist = lay.cap_hist;
     c.cap_spl = lay.cap_spl; c.cap_copy = lay.cap_copy; c.cap_ovf = lay.cap_ovf;
     c.seed = cfg.seed;
@@ -344,6 +345,8 @@ struct Engine {
     for (int phase = 0; phase < 2; phase++) {
       for (int cls = (int)cfg.nclass - 1; cls >= 0; cls--) {
         switch (kClassCap[cls]) {
+          case 512: GSS_TRY(launch_class<512>(c, cfg, cls, di, s, prof, count, phase)); break;
+          case 1024: GSS_TRY(launch_class<1024>(c, cfg, cls, di, s, prof, count, phase)); break;
           case 2048: GSS_TRY(launch_class<2048>(c, cfg, cls, di, s, prof, count, phase)); break;
           case 4096: GSS_TRY(launch_class<4096>(c, cfg, cls, di, s, prof, count, phase)); break;
           case 8192: GSS_TRY(launch_class<8192>(c, cfg, cls, di, s, prof, count, phase)); break;
@@ -544,7 +547,7 @@ gss_status gss_default_params(uint32_t key_bytes, uint32_t val_bytes, gss_params
   out->k = 256;
   out->oversample = 30;
   out->small_threshold = (val_bytes && key_bytes + val_bytes > 8) ? 8192 : 16384;
-  out->tile = 16384;
+  out->tile = 32768;
   out->k_policy = 1;
   out->fill_div = 4;
   out->seed = 5489;

@@ -11,7 +11,7 @@
 
 namespace gss {
 
-constexpr int kNumClasses = 4;        // in-SM sort size classes (2K, 4K, 8K, 16K keys)
+constexpr int kNumClasses = 6;        // in-SM sort size classes (512 .. 16K keys)
 constexpr int kMaxLevels = 16;        // distribution levels launched at most
 constexpr uint32_t kFull = 0xffffffffu;
 
@@ -80,7 +80,7 @@ struct Ctx {
   uint32_t* scan_part;
   const Key* given_spl;              // MODE_PARTITION_BY
   uint32_t given_nspl;
-  uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0;
+  uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
   uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf;
   uint32_t cap_small[kNumClasses];
   uint32_t class_cap[kNumClasses];

@@ -82,8 +82,19 @@ __global__ void __launch_bounds__(kSampleThreads, 1) k_sample(Ctx<Key, Val, IdT>
     if (c.sample_cap / kb < a) a = c.sample_cap / kb;
     if (a < 1) a = 1;
     const uint32_t s = a * kb;
-    for (uint32_t j = threadIdx.x; j < s; j += kSampleThreads)
-      sk[phys(j)] = src[B.lo + sample_pos(c.seed, level, B.lo, j, B.m)];
+    for (uint32_t j0 = threadIdx.x; j0 < s; j0 += 8 * kSampleThreads) {   // 8 gathers in flight
+      Key g[8];
+#pragma unroll
+      for (int u = 0; u < 8; u++) {
+        const uint32_t j = j0 + u * kSampleThreads;
+        if (j < s) g[u] = src[B.lo + sample_pos(c.seed, level, B.lo, j, B.m)];
+      }
+#pragma unroll
+      for (int u = 0; u < 8; u++) {
+        const uint32_t j = j0 + u * kSampleThreads;
+        if (j < s) sk[phys(j)] = g[u];
+      }
+    }
     Sorter::sort(sk, nullptr, (int)s, less);
     bool dup = false;
     for (uint32_t i = threadIdx.x; i + 2 < kb; i += kSampleThreads)
@@ -327,114 +338,10 @@ __device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t s
   return old;
 }
 
-// One chunk of <= kChunk keys of a tile: stable rank by (bucket id, position),
-// reorder in shared memory, write each bucket's run with coalesced stores.
-template <bool FULL, class Key, class Val, class IdT>
-__device__ __forceinline__ void scatter_chunk(const Key* __restrict__ ks, const Val* __restrict__ vs,
-                                              const IdT* __restrict__ is, Key* __restrict__ kdst,
-                                              Val* __restrict__ vdst, uint32_t clen, uint32_t K, uint32_t kmax,
-                                              uint32_t* gbase, uint32_t* ctot, uint32_t* delta, uint32_t* wcnt,
-                                              uint32_t* s_warp, Key* skeys, Val* svals, IdT* sids) {
-  constexpr int NW = kScatterThreads / 32;
-  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  const uint32_t ltmask = lanemask_lt();
-  uint32_t* wc = wcnt + w * kmax;
-  for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
-  Key kk[kScatterIter];
-  Val vv[kScatterIter];
-  uint32_t iid[kScatterIter], peers[kScatterIter], old[kScatterIter];
-  const uint32_t q0 = w * (32 * kScatterIter) + lane;
-#pragma unroll
-  for (int it = 0; it < kScatterIter; it++) {
-    const uint32_t q = q0 + it * 32;
-    if (FULL || q < clen) {
-      kk[it] = ks[q];
-      iid[it] = is[q];
-      if constexpr (kHasVal<Val>) vv[it] = vs[q];
-    } else {
-      iid[it] = 0xffffffffu;
-    }
-  }
-  __syncwarp();
-  // peer masks (lanes holding the same bucket id) from one ballot per id bit
-  constexpr int NBITS = sizeof(IdT) == 1 ? 8 : 10;
-#pragma unroll
-  for (int it = 0; it < kScatterIter; it++) {
-    const uint32_t id = iid[it];
-    uint32_t pm = FULL ? kFull : __ballot_sync(kFull, id != 0xffffffffu);
-#pragma unroll
-    for (int bit = 0; bit < NBITS; bit++) {
-      const bool on = (id >> bit) & 1u;
-      const uint32_t bal = __ballot_sync(kFull, on);
-      pm &= on ? bal : ~bal;
-    }
-    peers[it] = pm;
-  }
-  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
-#pragma unroll
-  for (int it = 0; it < kScatterIter; it++) {
-    // the lowest lane of each group of equal ids adds the group size to the
-    // warp's counter; ranks stay in lane order, hence stable (R7)
-    const uint32_t lead = ((FULL || iid[it] != 0xffffffffu) && (peers[it] & ltmask) == 0) ? 1u : 0u;
-    old[it] = atom_add_shared_if(lead, wc_s + 4 * (iid[it] & 0xffffu), (uint32_t)__popc(peers[it]));
-    __syncwarp();
-  }
-  uint32_t rk[kScatterIter];
-#pragma unroll
-  for (int it = 0; it < kScatterIter; it++)
-    rk[it] = __popc(peers[it] & ltmask) + __shfl_sync(kFull, old[it], __ffs(peers[it]) - 1);
-  __syncthreads();
-  // chunk totals per id, exclusive scan over ids, then every warp's start
-  // within each id folded into its counter (one lookup per key below)
-  const uint32_t per = (K + kScatterThreads - 1) / kScatterThreads;
-  const uint32_t i0 = threadIdx.x * per;
-  uint32_t tsum = 0;
-  for (uint32_t j = 0; j < per; j++) {
-    const uint32_t id = i0 + j;
-    if (id < K) {
-      uint32_t t = 0;
-#pragma unroll
-      for (int q = 0; q < NW; q++) t += wcnt[q * kmax + id];
-      ctot[id] = t;
-      tsum += t;
-    }
-  }
-  uint32_t ex = block_exclusive_scan<kScatterThreads>(tsum, s_warp, nullptr);
-  for (uint32_t j = 0; j < per; j++) {
-    const uint32_t id = i0 + j;
-    if (id < K) {
-      uint32_t run = ex;
-#pragma unroll
-      for (int q = 0; q < NW; q++) {
-        const uint32_t x = wcnt[q * kmax + id];
-        wcnt[q * kmax + id] = run;
-        run += x;
-      }
-      delta[id] = gbase[id] - ex;                         // global = delta + staged position
-      gbase[id] += ctot[id];
-      ex = run;
-    }
-  }
-  __syncthreads();
-#pragma unroll
-  for (int it = 0; it < kScatterIter; it++) {
-    if (FULL || iid[it] != 0xffffffffu) {
-      const uint32_t pos = wc[iid[it]] + rk[it];
-      skeys[pos] = kk[it];
-      if constexpr (kHasVal<Val>) svals[pos] = vv[it];
-      sids[pos] = (IdT)iid[it];
-    }
-  }
-  __syncthreads();
-#pragma unroll 4
-  for (uint32_t q = threadIdx.x; q < (FULL ? (uint32_t)kChunk : clen); q += kScatterThreads) {
-    const uint32_t d = delta[sids[q]] + q;
-    kdst[d] = skeys[q];
-    if constexpr (kHasVal<Val>) vdst[d] = svals[q];
-  }
-  __syncthreads();
-}
-
+// Phase 4 kernel.  Persistent: the CTA walks its tiles (blockIdx.x, +gridDim.x,
+// ...) chunk by chunk; the keys, values and ids of the next chunk are loaded
+// into registers before the current chunk's runs are written out, so the
+// global-load latency overlaps the write phase and the barriers.
 template <class Key, class Val, class IdT, class Cmp>
 __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
@@ -459,28 +366,175 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
   const Val* vsrc = nullptr;
   Val* vdst = nullptr;
   if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
+  const IdT* idsrc = c.ids;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  const uint32_t ltmask = lanemask_lt();
+  const bool stable = c.stable != 0;
+  uint32_t* wc = wcnt + w * kmax;
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
+  const uint32_t q0 = w * (32 * kScatterIter) + lane;
 
-  for (uint32_t t = blockIdx.x; t < nt; t += gridDim.x) {
-    const uint32_t b = c.tile_bucket[slot][t];
+  uint32_t t = blockIdx.x;
+  if (t >= nt) return;
+  // tile state
+  auto tile_info = [&](uint32_t tt, uint32_t& beg, uint32_t& len, uint32_t& K, uint32_t& hrow, uint32_t& hstride,
+                       uint32_t& tl, uint32_t& lo) {
+    const uint32_t b = c.tile_bucket[slot][tt];
     const Bucket B = c.bk[slot][b];
-    const uint32_t tl = t - B.tile_start;
-    const uint32_t beg = B.lo + tl * c.T;
-    const uint32_t len = min(c.T, B.m - tl * c.T);
-    const uint32_t* hist = c.hist[slot] + B.hist_base;
+    tl = tt - B.tile_start;
+    beg = B.lo + tl * c.T;
+    len = min(c.T, B.m - tl * c.T);
+    K = B.K;
+    hrow = B.hist_base;
+    hstride = B.ntiles;
+    lo = B.lo;
+  };
+  uint32_t beg, len, K, hrow, hstride, tl, blo;
+  tile_info(t, beg, len, K, hrow, hstride, tl, blo);
+  {
+    const uint32_t* hist = c.hist[slot] + hrow;
     const uint32_t hb = hist[0];
-    for (uint32_t id = threadIdx.x; id < B.K; id += kScatterThreads) gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
-    for (uint32_t c0 = 0; c0 < len; c0 += kChunk) {
-      const uint32_t clen = min((uint32_t)kChunk, len - c0);
-      const Key* ks = ksrc + beg + c0;
-      const Val* vs = nullptr;
-      if constexpr (kHasVal<Val>) vs = vsrc + beg + c0;
-      const IdT* is = c.ids + beg + c0;
-      if (clen == (uint32_t)kChunk)
-        scatter_chunk<true>(ks, vs, is, kdst, vdst, clen, B.K, kmax, gbase, ctot, delta, wcnt, s_warp, skeys, svals,
-                            sids);
-      else
-        scatter_chunk<false>(ks, vs, is, kdst, vdst, clen, B.K, kmax, gbase, ctot, delta, wcnt, s_warp, skeys, svals,
-                             sids);
+    for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
+  }
+  // prefetch registers: the chunk to process next
+  Key pk[kScatterIter];
+  Val pv[kScatterIter];
+  uint32_t pid[kScatterIter];
+  auto load_chunk = [&](uint32_t cbeg, uint32_t clen) {
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      const uint32_t q = q0 + it * 32;
+      pid[it] = 0xffffffffu;
+      if (q < clen) {
+        pk[it] = ksrc[cbeg + q];
+        pid[it] = idsrc[cbeg + q];
+        if constexpr (kHasVal<Val>) pv[it] = vsrc[cbeg + q];
+      }
+    }
+  };
+  uint32_t c0 = 0;
+  load_chunk(beg, min((uint32_t)kChunk, len));
+  for (;;) {
+    const uint32_t clen = min((uint32_t)kChunk, len - c0);
+    Key kk[kScatterIter];
+    Val vv[kScatterIter];
+    uint32_t iid[kScatterIter], rk[kScatterIter];
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      kk[it] = pk[it];
+      iid[it] = pid[it];
+      if constexpr (kHasVal<Val>) vv[it] = pv[it];
+    }
+    for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
+    __syncwarp();
+    if (stable) {
+      // Stable ranks (R7): peer masks of lanes holding the same bucket id, one
+      // ballot per id bit; the lowest lane of each group adds the group size to
+      // the warp's counter, so ranks follow lane order.
+      constexpr int NBITS = sizeof(IdT) == 1 ? 8 : 10;
+      uint32_t peers[kScatterIter], old[kScatterIter];
+#pragma unroll
+      for (int it = 0; it < kScatterIter; it++) {
+        const uint32_t id = iid[it];
+        uint32_t pm = __ballot_sync(kFull, id != 0xffffffffu);
+#pragma unroll
+        for (int bit = 0; bit < NBITS; bit++) {
+          const bool on = (id >> bit) & 1u;
+          const uint32_t bal = __ballot_sync(kFull, on);
+          pm &= on ? bal : ~bal;
+        }
+        peers[it] = pm;
+      }
+#pragma unroll
+      for (int it = 0; it < kScatterIter; it++) {
+        const uint32_t lead = (iid[it] != 0xffffffffu && (peers[it] & ltmask) == 0) ? 1u : 0u;
+        old[it] = atom_add_shared_if(lead, wc_s + 4 * (iid[it] & 0xffffu), (uint32_t)__popc(peers[it]));
+        __syncwarp();
+      }
+#pragma unroll
+      for (int it = 0; it < kScatterIter; it++)
+        rk[it] = __popc(peers[it] & ltmask) + __shfl_sync(kFull, old[it], __ffs(peers[it]) - 1);
+    } else {
+      // One shared-memory atomic per key on the warp's own counters: ranks are
+      // unique within (warp, id) in any order, so the level is a partition
+      // whose within-bucket order is the hardware's atomic order.
+#pragma unroll
+      for (int it = 0; it < kScatterIter; it++)
+        rk[it] = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (iid[it] & 0xffffu), 1u);
+    }
+    __syncthreads();
+    // chunk totals per id, exclusive scan over ids, then every warp's start
+    // within each id folded into its counter (one lookup per key below)
+    {
+      const uint32_t per = (K + kScatterThreads - 1) / kScatterThreads;
+      const uint32_t i0 = threadIdx.x * per;
+      uint32_t tsum = 0;
+      for (uint32_t j = 0; j < per; j++) {
+        const uint32_t id = i0 + j;
+        if (id < K) {
+          uint32_t tt = 0;
+#pragma unroll
+          for (int q = 0; q < NW; q++) tt += wcnt[q * kmax + id];
+          ctot[id] = tt;
+          tsum += tt;
+        }
+      }
+      uint32_t ex = block_exclusive_scan<kScatterThreads>(tsum, s_warp, nullptr);
+      for (uint32_t j = 0; j < per; j++) {
+        const uint32_t id = i0 + j;
+        if (id < K) {
+          uint32_t run = ex;
+#pragma unroll
+          for (int q = 0; q < NW; q++) {
+            const uint32_t x = wcnt[q * kmax + id];
+            wcnt[q * kmax + id] = run;
+            run += x;
+          }
+          delta[id] = gbase[id] - ex;                         // global index = delta + staged position
+          gbase[id] += ctot[id];
+          ex = run;
+        }
+      }
+    }
+    __syncthreads();
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      if (iid[it] != 0xffffffffu) {
+        const uint32_t pos = wc[iid[it]] + rk[it];
+        skeys[pos] = kk[it];
+        if constexpr (kHasVal<Val>) svals[pos] = vv[it];
+        sids[pos] = (IdT)iid[it];
+      }
+    }
+    __syncthreads();
+    // advance and prefetch the next chunk (possibly of the next tile)
+    const uint32_t cur_clen = clen;
+    bool new_tile = false;
+    bool done = false;
+    c0 += kChunk;
+    if (c0 >= len) {
+      t += gridDim.x;
+      c0 = 0;
+      if (t >= nt) done = true;
+      else {
+        tile_info(t, beg, len, K, hrow, hstride, tl, blo);
+        new_tile = true;
+      }
+    }
+    if (!done) load_chunk(beg + c0, min((uint32_t)kChunk, len - c0));
+    // write this chunk's bucket runs
+#pragma unroll 4
+    for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
+      const uint32_t d = delta[sids[q]] + q;
+      kdst[d] = skeys[q];
+      if constexpr (kHasVal<Val>) vdst[d] = svals[q];
+    }
+    __syncthreads();
+    if (done) break;
+    if (new_tile) {
+      const uint32_t* hist = c.hist[slot] + hrow;
+      const uint32_t hb = hist[0];
+      for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
     }
   }
 }
@@ -639,11 +693,29 @@ __global__ void __launch_bounds__(NT, (1024 / NT) > 0 ? 1024 / NT : 1)
   const Item* list = retry ? c.retry[cls] : c.small[cls];
   for (uint32_t i = blockIdx.x; i < ni; i += gridDim.x) {
     const Item I = list[i];
-    const Key* src = c.keys(I.buf);
-    for (uint32_t q = threadIdx.x; q < I.m; q += NT) sk[phys(q)] = src[I.lo + q];
-    if constexpr (kHasVal<Val>) {
-      const Val* vs = c.vals(I.buf);
-      for (uint32_t q = threadIdx.x; q < I.m; q += NT) sv[phys(q)] = vs[I.lo + q];
+    // load the bucket with ITEMS independent loads in flight per thread
+    const Key* src = c.keys(I.buf) + I.lo;
+    const Val* vs = nullptr;
+    if constexpr (kHasVal<Val>) vs = c.vals(I.buf) + I.lo;
+    for (uint32_t q0 = threadIdx.x; q0 < I.m; q0 += Sorter::ITEMS * NT) {
+      Key tk[Sorter::ITEMS];
+      Val tv[Sorter::ITEMS];
+#pragma unroll
+      for (int u = 0; u < Sorter::ITEMS; u++) {
+        const uint32_t q = q0 + u * NT;
+        if (q < I.m) {
+          tk[u] = src[q];
+          if constexpr (kHasVal<Val>) tv[u] = vs[q];
+        }
+      }
+#pragma unroll
+      for (int u = 0; u < Sorter::ITEMS; u++) {
+        const uint32_t q = q0 + u * NT;
+        if (q < I.m) {
+          sk[phys(q)] = tk[u];
+          if constexpr (kHasVal<Val>) sv[phys(q)] = tv[u];
+        }
+      }
     }
     Sorter::sort(sk, sv, (int)I.m, less);
     for (uint32_t q = threadIdx.x; q < I.m; q += NT) c.kout[I.lo + q] = sk[phys(q)];

@@ -252,3 +252,18 @@ def test_distributed_sorter_single_rank_nccl(gss):
     finally:
         if own:
             dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+def test_stable_flag_same_keys(gss, width, pairs):
+    """GSS_FLAG_STABLE (ballot-ranked stable scatter) and the default atomic-ranked scatter agree on keys."""
+    n = (1 << 20) + 3
+    x = inputs.keys("and2", n, width, seed=4)
+    v = inputs.values(n, width) if pairs else None
+    a = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=4)
+    b = gss.sort(to_dev(x), to_dev(v) if pairs else None)
+    np.testing.assert_array_equal(to_host(a[0]), to_host(b[0]))
+    np.testing.assert_array_equal(to_host(a[0]), np.sort(x))
+    if pairs:
+        check_pairs(x, to_host(a[1]), np.sort(x))
+        check_pairs(x, to_host(b[1]), np.sort(x))

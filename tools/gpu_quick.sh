@@ -10,4 +10,5 @@ timeout 600 python bench.py --workload $WL --no-cpu-baseline > gpurun_out/bench_
 echo "bench rc=$?"
 timeout 600 ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum --clock-control none --csv \
    --log-file gpurun_out/launches_${TAG}_${WL}.csv python tools/one_sort.py --workload $WL --warmup 1 --steps 1 > gpurun_out/launches_${TAG}.log 2>&1
+cp paper_conf_ipps_leischneros10_b200/libgss.so gpurun_out/libgss_${TAG}.so
 if [ -n "$4" ]; then tools/ncu_one.sh $TAG $4 ${5:-0} $WL; fi

@@ -19,13 +19,14 @@ ap.add_argument("--warmup", type=int, default=1)
 ap.add_argument("--k", type=int, default=256)
 ap.add_argument("--tile", type=int, default=16384)
 ap.add_argument("--M", type=int, default=0)
+ap.add_argument("--fill_div", type=int, default=0)
 args = ap.parse_args()
 n, bits, pairs, dist, _ = bench.WORKLOADS[args.workload]
 x = inputs.keys(dist, n, bits, seed=1)
 k = torch.from_numpy(x).cuda()
 v = torch.from_numpy(inputs.values(n, bits)).cuda() if pairs else None
 M = args.M or (8192 if (pairs and bits == 64) else 16384)
-s = gss.Sorter(f"u{bits}", n, pairs, k=args.k, tile=args.tile, M=M)
+s = gss.Sorter(f"u{bits}", n, pairs, k=args.k, tile=args.tile, M=M, fill_div=args.fill_div or None)
 ko = torch.empty_like(k)
 vo = torch.empty_like(v) if pairs else None
 for i in range(args.warmup + args.steps):
