@@ -178,6 +178,7 @@ def run_reference(args, wl):
 # our arm
 # ---------------------------------------------------------------------------
 def run_ours(args, wl):
+    os.environ.setdefault("NCCL_DEBUG", "WARN")          # keep stdout to the one JSON line
     import torch
     import torch.distributed as dist_mod
 
