@@ -107,6 +107,9 @@ typedef struct gss_params {
                                       partition); default: one shared atomic per key, which
                                       partitions correctly but orders keys within a bucket in
                                       the hardware's atomic order                             */
+#define GSS_FLAG_DIRECT_SCATTER 8u /* Phase 4 as in the paper: keys written straight from
+                                      registers at atomic-cursor positions, no smem reorder
+                                      (ablation, slower on B200)                  */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets with one more sample-sort split inside
                                       shared memory + warp merge sorts (P:332-335 variant)  */
 

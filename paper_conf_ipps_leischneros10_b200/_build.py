@@ -13,7 +13,7 @@ SOURCES = [os.path.join(CSRC, "gss.cu")]
 DEPS = SOURCES + [os.path.join(CSRC, f) for f in ("gss_device.cuh", "gss_kernels.cuh")] + [
     os.path.join(ROOT, "include", "gss.h")]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
-FLAGS = ["-gencode", "arch=compute_100a,code=sm_100a", "-O3", "-lineinfo", "-std=c++17",
+FLAGS = ["-gencode", "arch=compute_100a,code=sm_100a", "-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr",
          "-Xcompiler", "-fPIC", "-shared", "-Xptxas", "-v"]
 
 

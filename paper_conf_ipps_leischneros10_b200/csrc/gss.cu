@@ -270,7 +270,7 @@ struct Engine {
                                  gss_profiler* prof, uint32_t* count, uint32_t retry) {
     constexpr int NT = small_threads<Key, Val, CAP>();
     auto kern = k_small<Key, Val, IdT, Cmp, CAP>;
-    const size_t smem = CtaSort<Key, Val, NT, Cmp>::smem_bytes();
+    const size_t smem = CtaSort<Key, Val, NT, Cmp, small_items<Key, Val, CAP>()>::smem_bytes();
     GSS_TRY(set_smem(kern, smem));
     static int grid = 0;
     if (!grid) grid = grid_for(kern, NT, smem, di.sms);
@@ -324,6 +324,10 @@ struct Engine {
     if (!g_plan) g_plan = grid_for(k_plan<Key, Val, IdT>, kPlanThreads, 0, di.sms);
     const int g_cls = grid_for(kc, kClsThreads, sm_cls, di.sms);
     const int g_sc = grid_for(ksc, kScatterThreads, sm_sc, di.sms);
+    auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
+    const size_t sm_sd = (size_t)kmax * 4;
+    GSS_TRY(set_smem(ksd, sm_sd));
+    const int g_sd = grid_for(ksd, kDirectThreads, sm_sd, di.sms);
     for (uint32_t l = 0; l < c.L; l++) {
       if (mode == MODE_PARTITION_BY) {
         GSS_TRY(launch(prof, GSS_K_SAMPLE, s, count, [&] { k_set_splitters<Key, Val, IdT><<<1, 256, 0, s>>>(c); }));
@@ -335,7 +339,12 @@ struct Engine {
                      [&] { k_scan_reduce<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
       GSS_TRY(launch(prof, GSS_K_SCAN, s, count,
                      [&] { k_scan_final<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
-      GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));
+      if (!(cfg.flags & GSS_FLAG_DIRECT_SCATTER) || c.stable) {
+        GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));
+      } else {
+        GSS_TRY(launch(prof, GSS_K_SCATTER, s, count,
+                       [&] { ksd<<<g_sd, kDirectThreads, sm_sd, s>>>(c, l); }));
+      }
       if (mode == MODE_SORT)
         GSS_TRY(launch(prof, GSS_K_PLAN, s, count, [&] { k_plan<Key, Val, IdT><<<g_plan, kPlanThreads, 0, s>>>(c, l); }));
     }

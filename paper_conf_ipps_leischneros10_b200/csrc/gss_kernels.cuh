@@ -539,6 +539,81 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
   }
 }
 
+// Phase 4 as the paper describes it: every key goes
+// straight from registers to its global position; the position is the tile's
+// offset for its bucket plus a shared-memory atomic cursor (the per-block
+// counters of P:312-317).  No staging and no barriers inside a tile; the
+// within-bucket order is the atomics' order (a valid partition, not stable).
+// A warp whose 32 keys share one bucket (sorted input) takes one atomic.
+constexpr int kDirectThreads = 256;
+template <class Key, class Val, class IdT, class Cmp>
+__global__ void __launch_bounds__(kDirectThreads, 4) k_scatter_direct(Ctx<Key, Val, IdT> c, uint32_t level) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  uint32_t* cursor = reinterpret_cast<uint32_t*>(smem_raw);
+  const uint32_t cur_s = (uint32_t)__cvta_generic_to_shared(cursor);
+  const uint32_t slot = level & 1;
+  const uint32_t nt = c.cnt->lvl[level].num_tiles;
+  const uint32_t sb = c.src(level), db = c.dst(level);
+  const Key* ksrc = c.keys(sb);
+  Key* kdst = c.wkeys(db);
+  const Val* vsrc = nullptr;
+  Val* vdst = nullptr;
+  if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
+  const int lane = threadIdx.x & 31;
+  const uint32_t ltmask = lanemask_lt();
+  constexpr int U = 8;
+  for (uint32_t t = blockIdx.x; t < nt; t += gridDim.x) {
+    const uint32_t b = c.tile_bucket[slot][t];
+    const Bucket B = c.bk[slot][b];
+    const uint32_t tl = t - B.tile_start;
+    const uint32_t beg = B.lo + tl * c.T;
+    const uint32_t len = min(c.T, B.m - tl * c.T);
+    const uint32_t* hist = c.hist[slot] + B.hist_base;
+    const uint32_t hb = hist[0];
+    __syncthreads();
+    for (uint32_t id = threadIdx.x; id < B.K; id += kDirectThreads) cursor[id] = hist[id * B.ntiles + tl] - hb + B.lo;
+    __syncthreads();
+    const Key* ks = ksrc + beg;
+    const IdT* is = c.ids + beg;
+    const Val* vs = nullptr;
+    if constexpr (kHasVal<Val>) vs = vsrc + beg;
+    for (uint32_t w0 = threadIdx.x & ~31u; w0 < len; w0 += U * kDirectThreads) {   // warp-uniform trip count
+      const uint32_t i0 = w0 + lane;
+      Key kk[U];
+      Val vv[U];
+      uint32_t id[U];
+#pragma unroll
+      for (int u = 0; u < U; u++) {
+        const uint32_t i = i0 + u * kDirectThreads;
+        id[u] = 0xffffffffu;
+        if (i < len) {
+          kk[u] = ks[i];
+          id[u] = is[i];
+          if constexpr (kHasVal<Val>) vv[u] = vs[i];
+        }
+      }
+#pragma unroll
+      for (int u = 0; u < U; u++) {
+        const uint32_t myid = id[u];
+        const uint32_t first = __shfl_sync(kFull, myid, 0);
+        uint32_t d;
+        if (__all_sync(kFull, myid == first) && first != 0xffffffffu) {
+          // the whole warp in one bucket: one atomic, lane order
+          uint32_t base = 0;
+          if (lane == 0) base = atomicAdd(&cursor[first], 32u);
+          d = __shfl_sync(kFull, base, 0) + (uint32_t)__popc(ltmask);
+        } else {
+          d = atom_add_shared_if(myid != 0xffffffffu ? 1u : 0u, cur_s + 4 * (myid & 0xffffu), 1u);
+        }
+        if (myid != 0xffffffffu) {
+          kdst[d] = kk[u];
+          if constexpr (kHasVal<Val>) vdst[d] = vv[u];
+        }
+      }
+    }
+  }
+}
+
 // ---------------------------------------------------------------------------
 // Recursion (Algorithm 1) with delayed small sorts: every
 // child of every bucket split at this level becomes a next-level bucket
@@ -678,14 +753,25 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
 // Sorting buckets: one CTA per bucket of at most M keys; the
 // bucket is loaded to shared memory, sorted by CtaSort, written to keys_out.
 // ---------------------------------------------------------------------------
+// keys per thread of the bucket sorter (32 items per thread measured slower
+// on B200: register pressure outweighs the saved merge round), i.e. the
+// CtaSort default
 template <class Key, class Val, int CAP>
-constexpr int small_threads() { return CAP / sort_items<Key, Val>(); }
+constexpr int small_items() { return sort_items<Key, Val>(); }
+template <class Key, class Val, int CAP>
+constexpr int small_threads() { return CAP / small_items<Key, Val, CAP>(); }
+
+template <class Key, class Val, int CAP, int NT>
+constexpr int small_min_blocks() {
+  // 64 registers per thread (16 items), 128 with 32 items
+  return ((small_items<Key, Val, CAP>() >= 32 ? 512 : 1024) / NT) > 0 ? (small_items<Key, Val, CAP>() >= 32 ? 512 : 1024) / NT : 1;
+}
 
 template <class Key, class Val, class IdT, class Cmp, int CAP, int NT = small_threads<Key, Val, CAP>()>
-__global__ void __launch_bounds__(NT, (1024 / NT) > 0 ? 1024 / NT : 1)
+__global__ void __launch_bounds__(NT, small_min_blocks<Key, Val, CAP, NT>())
     k_small(Ctx<Key, Val, IdT> c, uint32_t cls, uint32_t retry) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  using Sorter = CtaSort<Key, Val, NT, Cmp>;
+  using Sorter = CtaSort<Key, Val, NT, Cmp, small_items<Key, Val, CAP>()>;
   Key* sk = reinterpret_cast<Key*>(smem_raw);
   Val* sv = reinterpret_cast<Val*>(smem_raw + (size_t)Sorter::PL * sizeof(Key));
   const Cmp less;
@@ -697,11 +783,12 @@ __global__ void __launch_bounds__(NT, (1024 / NT) > 0 ? 1024 / NT : 1)
     const Key* src = c.keys(I.buf) + I.lo;
     const Val* vs = nullptr;
     if constexpr (kHasVal<Val>) vs = c.vals(I.buf) + I.lo;
-    for (uint32_t q0 = threadIdx.x; q0 < I.m; q0 += Sorter::ITEMS * NT) {
-      Key tk[Sorter::ITEMS];
-      Val tv[Sorter::ITEMS];
+    constexpr int LU = 4;                                  // loads in flight per thread
+    for (uint32_t q0 = threadIdx.x; q0 < I.m; q0 += LU * NT) {
+      Key tk[LU];
+      Val tv[LU];
 #pragma unroll
-      for (int u = 0; u < Sorter::ITEMS; u++) {
+      for (int u = 0; u < LU; u++) {
         const uint32_t q = q0 + u * NT;
         if (q < I.m) {
           tk[u] = src[q];
@@ -709,7 +796,7 @@ __global__ void __launch_bounds__(NT, (1024 / NT) > 0 ? 1024 / NT : 1)
         }
       }
 #pragma unroll
-      for (int u = 0; u < Sorter::ITEMS; u++) {
+      for (int u = 0; u < LU; u++) {
         const uint32_t q = q0 + u * NT;
         if (q < I.m) {
           sk[phys(q)] = tk[u];

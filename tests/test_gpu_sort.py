@@ -267,3 +267,15 @@ def test_stable_flag_same_keys(gss, width, pairs):
     if pairs:
         check_pairs(x, to_host(a[1]), np.sort(x))
         check_pairs(x, to_host(b[1]), np.sort(x))
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+def test_direct_scatter_ablation(gss, width, pairs):
+    """GSS_FLAG_DIRECT_SCATTER (the paper's unstructured Phase 4) sorts correctly."""
+    n = (1 << 20) + 11
+    x = inputs.keys("staggered", n, width, seed=3)
+    v = inputs.values(n, width) if pairs else None
+    ko, vo = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=8)
+    np.testing.assert_array_equal(to_host(ko), np.sort(x))
+    if pairs:
+        check_pairs(x, to_host(vo), np.sort(x))
