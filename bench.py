@@ -196,7 +196,7 @@ def run_ours(args, wl):
     wk = bits // 8
     wv = wk if pairs else 0
     kind = f"u{bits}"
-    params = dict(k=256, a=30, tile=32768)
+    params = dict(k=256, a=30, tile=32768, flags=16)            # flags 16: replay the launch sequence as a CUDA graph
     if wl == "c1_u32_2p16":
         params.update(k=128, k_policy="fixed")
     M = 8192 if (pairs and bits == 64) else 16384

@@ -110,6 +110,10 @@ typedef struct gss_params {
 #define GSS_FLAG_DIRECT_SCATTER 8u /* Phase 4 as in the paper: keys written straight from
                                       registers at atomic-cursor positions, no smem reorder
                                       (ablation, slower on B200)                  */
+#define GSS_FLAG_GRAPH 16u         /* capture the launch sequence of a device-buffer sort as a
+                                      CUDA graph on first use and replay it on later calls
+                                      with identical buffers, n and parameters (launch-bound
+                                      sizes); ignored with stats or a profiler              */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets with one more sample-sort split inside
                                       shared memory + warp merge sorts (P:332-335 variant)  */
 

@@ -396,6 +396,51 @@ void fill_stats(const Counters& h, uint32_t L, uint32_t launches, gss_stats* st)
   st->overflow_elems = h.ovf_elems;
 }
 
+// Cache of instantiated launch graphs (GSS_FLAG_GRAPH), keyed by everything
+// the captured kernels bake in: entry point, device, n, buffers, parameters.
+struct GraphKey {
+  const void* fn;
+  int dev;
+  uint64_t n;
+  const void* p[5];
+  uint32_t cfg[8];
+  uint64_t seed;
+  bool operator==(const GraphKey& o) const { return memcmp(this, &o, sizeof(GraphKey)) == 0; }
+};
+struct GraphEntry {
+  GraphKey key;
+  cudaGraphExec_t exec;
+};
+std::mutex g_graph_mu;
+std::vector<GraphEntry> g_graphs;
+constexpr size_t kGraphCacheSize = 16;
+
+cudaStream_t capture_stream(int dev) {
+  static cudaStream_t streams[64] = {};
+  std::lock_guard<std::mutex> g(g_graph_mu);
+  if (dev < 0 || dev >= 64) return nullptr;
+  if (!streams[dev] && cudaStreamCreateWithFlags(&streams[dev], cudaStreamNonBlocking) != cudaSuccess) {
+    cudaGetLastError();
+    streams[dev] = nullptr;
+  }
+  return streams[dev];
+}
+
+cudaGraphExec_t graph_lookup(const GraphKey& k) {
+  std::lock_guard<std::mutex> g(g_graph_mu);
+  for (auto& e : g_graphs)
+    if (e.key == k) return e.exec;
+  return nullptr;
+}
+void graph_insert(const GraphKey& k, cudaGraphExec_t exec) {
+  std::lock_guard<std::mutex> g(g_graph_mu);
+  if (g_graphs.size() >= kGraphCacheSize) {
+    cudaGraphExecDestroy(g_graphs.front().exec);
+    g_graphs.erase(g_graphs.begin());
+  }
+  g_graphs.push_back({k, exec});
+}
+
 // Shared driver of every entry point.
 struct IO {
   const void* kin; const void* vin; void* kout; void* vout;
@@ -487,6 +532,45 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
       }
       c.given_spl = reinterpret_cast<const Key*>(io.given_spl);
       c.given_nspl = io.given_nspl;
+    }
+    if ((cfg.flags & GSS_FLAG_GRAPH) && mode == MODE_SORT && !host_io && !prof && !(up && up->stats)) {
+      // replay (or capture once) the whole launch sequence as a CUDA graph
+      GraphKey key;
+      memset(&key, 0, sizeof(key));
+      key.fn = reinterpret_cast<const void*>(&Eng::run);
+      key.dev = di.dev;
+      key.n = n;
+      key.p[0] = io.kin; key.p[1] = io.kout; key.p[2] = io.vin; key.p[3] = io.vout; key.p[4] = temp;
+      key.cfg[0] = cfg.k; key.cfg[1] = cfg.a; key.cfg[2] = cfg.T; key.cfg[3] = cfg.L; key.cfg[4] = cfg.k_policy;
+      key.cfg[5] = cfg.fill_div; key.cfg[6] = cfg.flags; key.cfg[7] = (uint32_t)cfg.M;
+      key.seed = cfg.seed;
+      cudaGraphExec_t exec = graph_lookup(key);
+      if (!exec) {
+        // capture on a private non-blocking stream (the caller's may be the legacy
+        // default stream, which cannot be captured); the graph replays on `s`
+        cudaGraph_t g = nullptr;
+        cudaStream_t cs = capture_stream(di.dev);
+        if (!cs || cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal) != cudaSuccess) {
+          cudaGetLastError();
+          return GSS_ERROR_CUDA;
+        }
+        const gss_status st = Eng::run(c, cfg, mode, di, cs, nullptr, &count);
+        const cudaError_t ce = cudaStreamEndCapture(cs, &g);
+        if (st != GSS_SUCCESS || ce != cudaSuccess) {
+          cudaGetLastError();
+          if (g) cudaGraphDestroy(g);
+          return st != GSS_SUCCESS ? st : GSS_ERROR_CUDA;
+        }
+        if (cudaGraphInstantiate(&exec, g, 0) != cudaSuccess) {
+          cudaGetLastError();
+          cudaGraphDestroy(g);
+          return GSS_ERROR_CUDA;
+        }
+        cudaGraphDestroy(g);
+        graph_insert(key, exec);
+      }
+      if (cudaGraphLaunch(exec, s) != cudaSuccess) { cudaGetLastError(); return GSS_ERROR_CUDA; }
+      return GSS_SUCCESS;
     }
     GSS_TRY(Eng::run(c, cfg, mode, di, s, prof, &count));
     if (mode != MODE_SORT) {
