@@ -191,6 +191,27 @@ __device__ __forceinline__ uint64_t block_sum_u64(uint64_t x, unsigned long long
 __host__ __device__ constexpr int padded_len(int c) { return c + c / 16 + 1; }
 __device__ __forceinline__ int phys(int i) { return i + (i >> 4); }
 
+// a = *p if pred, else b = *p: one predicated shared-memory load per target
+template <class T>
+__device__ __forceinline__ void load_pred(T& a, T& b, const T* p, bool pred) {
+  const uint32_t s = (uint32_t)__cvta_generic_to_shared(p);
+  if constexpr (sizeof(T) == 8) {
+    unsigned long long x = (unsigned long long)a, y = (unsigned long long)b;
+    asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.shared.u64 %0, [%3];\n\t"
+                 "@!q ld.shared.u64 %1, [%3];\n\t}"
+                 : "+l"(x), "+l"(y)
+                 : "r"((uint32_t)pred), "r"(s));
+    a = (T)x; b = (T)y;
+  } else if constexpr (sizeof(T) == 4) {
+    uint32_t x = (uint32_t)a, y = (uint32_t)b;
+    asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.shared.u32 %0, [%3];\n\t"
+                 "@!q ld.shared.u32 %1, [%3];\n\t}"
+                 : "+r"(x), "+r"(y)
+                 : "r"((uint32_t)pred), "r"(s));
+    a = (T)x; b = (T)y;
+  }
+}
+
 template <class Key, class Val, class Cmp>
 __device__ __forceinline__ void cmp_swap(Key& a, Key& b, Val& va, Val& vb, Cmp less) {
   bool s = less(b, a);
@@ -273,6 +294,24 @@ struct CtaSort {
     Key ka = sk[phys(ia)], kb = sk[phys(ib)];
     Val va, vb;
     if constexpr (kHasVal<Val>) { va = sv[phys(ia)]; vb = sv[phys(ib)]; }
+    if (__all_sync(__activemask(), ia + ITEMS <= ae && ib + ITEMS <= be)) {
+      // no lane can exhaust a run in its window: no bounds tests, and the next
+      // key is loaded straight into the register of the side that advanced
+#pragma unroll
+      for (int i = 0; i < ITEMS; i++) {
+        const bool p = !less(kb, ka);
+        k[i] = p ? ka : kb;
+        if constexpr (kHasVal<Val>) v[i] = p ? va : vb;
+        if (i + 1 < ITEMS) {
+          const int nx = (p ? ia : ib) + 1;
+          ia = p ? nx : ia;
+          ib = p ? ib : nx;
+          load_pred(ka, kb, sk + phys(nx), p);
+          if constexpr (kHasVal<Val>) load_pred(va, vb, sv + phys(nx), p);
+        }
+      }
+      return;
+    }
 #pragma unroll
     for (int i = 0; i < ITEMS; i++) {
       const bool p = (ib >= be) || (ia < ae && !less(kb, ka));
