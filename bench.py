@@ -35,6 +35,8 @@ import inputs  # noqa: E402
 WORKLOADS = {
     # name: (n, key bits, pairs, distribution, description)
     "c4_u64_2p28": (1 << 28, 64, False, "uniform", "2^28 uniform u64 keys (BASELINE configs[3], the north-star target row)"),
+    "c4_u64_2p29": (1 << 29, 64, False, "uniform", "2^29 uniform u64 keys (BASELINE configs[3] sweep)"),
+    "c4_u64_2p30": (1 << 30, 64, False, "uniform", "2^30 uniform u64 keys (BASELINE configs[3] sweep)"),
     "c2_u32_2p27": (1 << 27, 32, False, "uniform", "2^27 uniform u32 keys (BASELINE configs[1])"),
     "c3_u64_2p27": (1 << 27, 64, False, "uniform", "2^27 uniform u64 keys (BASELINE configs[2])"),
     "c3_kv64_2p27": (1 << 27, 64, True, "uniform", "2^27 uniform u64 key + u64 value pairs (BASELINE configs[2])"),
