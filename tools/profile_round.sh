@@ -7,7 +7,7 @@ mkdir -p gpurun_out
 timeout 600 ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum --clock-control none --csv \
    --log-file gpurun_out/launches_${TAG}_${WL}.csv python tools/one_sort.py --workload $WL --warmup 1 --steps 1 > gpurun_out/launches_${TAG}.log 2>&1
 echo "launches rc=$?"
-for spec in "k_classify:0" "k_scatter:0" "k_small:4"; do
+for spec in "k_classify:0" "k_scatter:0" "k_small:1"; do
   K=${spec%%:*}; S=${spec##*:}
   timeout 900 ncu --set full --clock-control none --import-source on -k regex:$K -s $S -c 1 \
      -o gpurun_out/prof_${TAG}_${K} -f python tools/one_sort.py --workload $WL --warmup 0 --steps 1 \
