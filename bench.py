@@ -285,7 +285,7 @@ def run_ours(args, wl):
         if os.path.exists(tpath):
             tr = json.load(open(tpath))
             if dom in tr:
-                traffic = tr[dom]
+                traffic = tr[dom]                      # DRAM bytes per step of this kernel kind (ncu)
         roof = {"bound": "hbm", "kernel": dom, "achieved": round(achieved, 1), "peak": hbm, "unit": "GB/s",
                 "frac": round(achieved / hbm, 4), "traffic": traffic, "alg_bytes_per_step": ab,
                 "launches_per_step": per[dom][1], "peak_source": peak_src}
