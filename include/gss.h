@@ -162,6 +162,22 @@ gss_status gss_sort_host_pairs_u64(const uint64_t* h_keys_in, const uint64_t* h_
                                    void* temp, size_t* temp_bytes, void* stream,
                                    const gss_params* p);
 
+/* Pipelined end-to-end sorting of a stream of host arrays of n elements:
+ * call i's host->device copy, the sort of call i-1 and the device->host copy
+ * of call i-2 overlap on three internal streams (two device buffer sets kept
+ * in temp).  Each run() is ordered after earlier work on `stream`; `stream`
+ * then waits for the PREVIOUS run's output (one-call lag), and flush() makes
+ * it wait for the last one, so after flush() + synchronising `stream` every
+ * output is valid.  key_bytes 4|8, val_bytes 0 or key_bytes.  temp == NULL
+ * queries *temp_bytes (no GPU access, *out untouched). */
+typedef struct gss_host_pipeline gss_host_pipeline;
+gss_status gss_host_pipeline_create(gss_host_pipeline** out, uint32_t key_bytes, uint32_t val_bytes, size_t n,
+                                    const gss_params* p, void* temp, size_t* temp_bytes);
+gss_status gss_host_pipeline_run(gss_host_pipeline* h, const void* h_keys_in, const void* h_vals_in,
+                                 void* h_keys_out, void* h_vals_out, void* stream);
+gss_status gss_host_pipeline_flush(gss_host_pipeline* h, void* stream);
+gss_status gss_host_pipeline_destroy(gss_host_pipeline* h);
+
 /* ---------------------------------------------------------------------- */
 /* One k-way distribution step over the whole input (Phases 1-4,           */
 /* P:251-263), regardless of M.  The partition is stable (R7).   */

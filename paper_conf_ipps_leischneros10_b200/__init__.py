@@ -19,7 +19,7 @@ import torch
 
 from . import _build
 
-__all__ = ["sort", "sort_host", "Sorter", "HostSorter", "partition", "partition_by", "sample", "Profiler", "Stats", "temp_bytes",
+__all__ = ["sort", "sort_host", "Sorter", "HostSorter", "HostPipeline", "partition", "partition_by", "sample", "Profiler", "Stats", "temp_bytes",
            "library_path", "KERNEL_KINDS"]
 
 KERNEL_KINDS = ["init", "sample", "classify", "scan", "scatter", "plan", "small_sort", "copy", "overflow", "h2d",
@@ -107,6 +107,14 @@ def _lib():
             f = getattr(lib, name)
             f.restype = ctypes.c_int
             f.argtypes = [_vp, _sz, _u64, _u32, _u64, _vp, _sz, _vp]
+        lib.gss_host_pipeline_create.restype = ctypes.c_int
+        lib.gss_host_pipeline_create.argtypes = [ctypes.POINTER(_vp), _u32, _u32, _sz, P, _vp, szp]
+        lib.gss_host_pipeline_run.restype = ctypes.c_int
+        lib.gss_host_pipeline_run.argtypes = [_vp, _vp, _vp, _vp, _vp, _vp]
+        lib.gss_host_pipeline_flush.restype = ctypes.c_int
+        lib.gss_host_pipeline_flush.argtypes = [_vp, _vp]
+        lib.gss_host_pipeline_destroy.restype = ctypes.c_int
+        lib.gss_host_pipeline_destroy.argtypes = [_vp]
         lib.gss_status_string.restype = ctypes.c_char_p
         lib.gss_status_string.argtypes = [ctypes.c_int]
         lib.gss_version.restype = _u32
@@ -314,6 +322,43 @@ class HostSorter:
             rc = self.fn(_ptr(h_keys), _ptr(h_out), self.n, _ptr(self.temp), ctypes.byref(tb), s, ctypes.byref(p))
         _check(rc, self.fn.__name__)
         return Stats._from(st) if stats else None
+
+
+class HostPipeline:
+    """Pipelined end-to-end sorts of host (pinned) arrays through gss_host_pipeline_*:
+    consecutive calls overlap host->device copy, sort and device->host copy."""
+
+    def __init__(self, kind: str, n: int, pairs: bool = False, device=None, **params):
+        self.lib = _lib()
+        self.n = n
+        self.device = torch.device(device or "cuda")
+        kb = 4 if kind == "u32" else 8
+        self._p = _params(**params)
+        tb = _sz(0)
+        _check(self.lib.gss_host_pipeline_create(None, kb, kb if pairs else 0, n, ctypes.byref(self._p), None,
+                                                 ctypes.byref(tb)), "gss_host_pipeline_create (query)")
+        self.temp = torch.empty(max(tb.value, 1), dtype=torch.uint8, device=self.device)
+        h = _vp()
+        _check(self.lib.gss_host_pipeline_create(ctypes.byref(h), kb, kb if pairs else 0, n, ctypes.byref(self._p),
+                                                 _ptr(self.temp), ctypes.byref(tb)), "gss_host_pipeline_create")
+        self._h = h
+
+    def __call__(self, h_keys, h_out, h_vals=None, h_vals_out=None, stream=None):
+        s = stream.cuda_stream if stream is not None else torch.cuda.current_stream(self.device).cuda_stream
+        _check(self.lib.gss_host_pipeline_run(self._h, _ptr(h_keys), _ptr(h_vals), _ptr(h_out), _ptr(h_vals_out), s),
+               "gss_host_pipeline_run")
+
+    def flush(self, stream=None):
+        """Make `stream` wait for the last run's output (then synchronise it)."""
+        s = stream.cuda_stream if stream is not None else torch.cuda.current_stream(self.device).cuda_stream
+        _check(self.lib.gss_host_pipeline_flush(self._h, s), "gss_host_pipeline_flush")
+
+    def __del__(self):
+        try:
+            if getattr(self, "_h", None) and _LIB is not None:
+                _LIB.gss_host_pipeline_destroy(self._h)
+        except Exception:
+            pass
 
 
 def sort_host(h_keys: torch.Tensor, h_values: torch.Tensor | None = None, **params):

@@ -292,3 +292,23 @@ def test_graph_replay(gss):
         kin.copy_(torch.from_numpy(x))
         s(kin, kout)
         np.testing.assert_array_equal(to_host(kout), np.sort(x))
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+def test_host_pipeline(gss, width, pairs):
+    """gss_host_pipeline_*: consecutive pipelined host-buffer sorts are each correct."""
+    n = (1 << 18) + 5
+    hp = gss.HostPipeline(f"u{width}", n, pairs)
+    xs = [inputs.keys("uniform", n, width, seed=s) for s in (1, 2, 3, 4)]
+    his = [torch.from_numpy(x).pin_memory() for x in xs]
+    hos = [torch.empty_like(h).pin_memory() for h in his]
+    hv = torch.from_numpy(inputs.values(n, width)).pin_memory() if pairs else None
+    hvo = [torch.empty_like(hv).pin_memory() for _ in xs] if pairs else [None] * 4
+    for i in range(4):
+        hp(his[i], hos[i], hv, hvo[i])
+    hp.flush()
+    torch.cuda.synchronize()
+    for i in range(4):
+        np.testing.assert_array_equal(hos[i].numpy(), np.sort(xs[i]))
+        if pairs:
+            check_pairs(xs[i], hvo[i].numpy(), np.sort(xs[i]))
