@@ -144,6 +144,14 @@ gss_status gss_sort_u64_descending(const uint64_t* keys_in, uint64_t* keys_out, 
                                    void* temp, size_t* temp_bytes, void* stream,
                                    const gss_params* p);
 
+/* Floating-point keys under the IEEE-754 total order (-NaN < -inf < ... < -0 <
+ * +0 < ... < +inf < +NaN): the same kernels with a different comparator
+ * (the paper sorts floats). */
+gss_status gss_sort_f32(const float* keys_in, float* keys_out, size_t n,
+                        void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_sort_f64(const double* keys_in, double* keys_out, size_t n,
+                        void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+
 /* End-to-end variants: keys (and values) are HOST buffers (pinned for full
  * speed); the call enqueues the host->device copy, the sort and the
  * device->host copy on `stream`.  temp must also hold the device copies

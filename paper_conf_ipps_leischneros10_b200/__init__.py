@@ -85,8 +85,8 @@ def _lib():
         lib = ctypes.CDLL(_build.LIB)
         P = ctypes.POINTER(_Params)
         szp = ctypes.POINTER(_sz)
-        for name in ("gss_sort_u32", "gss_sort_u64", "gss_sort_u64_descending", "gss_sort_host_u32",
-                     "gss_sort_host_u64"):
+        for name in ("gss_sort_u32", "gss_sort_u64", "gss_sort_u64_descending", "gss_sort_f32", "gss_sort_f64",
+                     "gss_sort_host_u32", "gss_sort_host_u64"):
             f = getattr(lib, name)
             f.restype = ctypes.c_int
             f.argtypes = [_vp, _vp, _sz, _vp, szp, _vp, P]
@@ -187,7 +187,11 @@ def _kind(t: torch.Tensor) -> str:
         return "u32"
     if t.dtype == torch.uint64:
         return "u64"
-    raise TypeError(f"keys must be torch.uint32 or torch.uint64, got {t.dtype}")
+    if t.dtype == torch.float32:
+        return "f32"
+    if t.dtype == torch.float64:
+        return "f64"
+    raise TypeError(f"keys must be torch.uint32, uint64, float32 or float64, got {t.dtype}")
 
 
 def _stream(t: torch.Tensor, stream):
@@ -210,7 +214,8 @@ def _temp(fn, args_before_temp, stream_and_params, device):
 def sort(keys: torch.Tensor, values: torch.Tensor | None = None, *, out: torch.Tensor | None = None,
          values_out: torch.Tensor | None = None, descending: bool = False, stats: bool = False,
          profiler: Profiler | None = None, stream=None, **params):
-    """Sort device keys (torch.uint32 / torch.uint64, CUDA) and optional values.
+    """Sort device keys (torch.uint32 / torch.uint64, CUDA) and optional values;
+    float32 / float64 keys (keys only) sort in IEEE-754 totalOrder.
 
     Returns (keys_out, values_out) or, with stats=True, (keys_out, values_out, Stats).
     params: k, M, a, tile, seed, k_policy ('adaptive'|'fixed'), fill_div, max_levels, flags."""
@@ -225,6 +230,8 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, *, out: torch.T
     p = _params(stats=st, profiler=profiler, **params)
     s = _stream(keys, stream)
     if values is not None:
+        if kind in ("f32", "f64"):
+            raise NotImplementedError("float keys are exported keys-only")
         if descending:
             raise NotImplementedError("descending order is exported for keys-only u64")
         values = values.contiguous()

@@ -1,43 +1,75 @@
-"""Build libgss.so (the CUDA sample sort behind include/gss.h) for sm_100a, in tree."""
+"""Build libgss.so (the CUDA sample sort behind include/gss.h) for sm_100a, in tree.
+
+Every translation unit in csrc/ (gss.cu: the C ABI; gss_inst_*.cu: one
+instantiation of the sort engine each) is compiled with
+`nvcc -gencode arch=compute_100a,code=sm_100a -O3 -lineinfo` in parallel, then
+linked into paper_conf_ipps_leischneros10_b200/libgss.so."""
 from __future__ import annotations
 
+import glob
 import os
 import subprocess
 import sys
+from concurrent.futures import ThreadPoolExecutor
 
 PKG = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
+OBJ = os.path.join(PKG, "build_obj")
 LIB = os.path.join(PKG, "libgss.so")
-SOURCES = [os.path.join(CSRC, "gss.cu")]
-DEPS = SOURCES + [os.path.join(CSRC, f) for f in ("gss_device.cuh", "gss_kernels.cuh")] + [
-    os.path.join(ROOT, "include", "gss.h")]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
-FLAGS = ["-gencode", "arch=compute_100a,code=sm_100a", "-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr",
-         "-Xcompiler", "-fPIC", "-shared", "-Xptxas", "-v"]
+ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
+FLAGS = ARCH + ["-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr", "-Xcompiler", "-fPIC",
+                "-Xptxas", "-v"]
+
+
+def sources():
+    return sorted(glob.glob(os.path.join(CSRC, "*.cu")))
+
+
+def deps():
+    return sources() + glob.glob(os.path.join(CSRC, "*.cuh")) + [os.path.join(ROOT, "include", "gss.h")]
 
 
 def stale() -> bool:
     if not os.path.exists(LIB):
         return True
     t = os.path.getmtime(LIB)
-    return any(os.path.getmtime(d) > t for d in DEPS)
+    return any(os.path.getmtime(d) > t for d in deps())
+
+
+def _compile(src: str):
+    obj = os.path.join(OBJ, os.path.basename(src)[:-3] + ".o")
+    cmd = [NVCC, *FLAGS, "-c", "-o", obj, src]
+    r = subprocess.run(cmd, capture_output=True, text=True)
+    return src, obj, cmd, r
 
 
 def build(force: bool = False, verbose: bool = False) -> str:
     if not force and not stale():
         return LIB
-    cmd = [NVCC, *FLAGS, "-o", LIB + ".tmp", *SOURCES]
-    r = subprocess.run(cmd, capture_output=True, text=True)
+    os.makedirs(OBJ, exist_ok=True)
+    srcs = sources()
+    with ThreadPoolExecutor(max_workers=min(len(srcs), os.cpu_count() or 4)) as ex:
+        results = list(ex.map(_compile, srcs))
     log = os.path.join(PKG, "build.log")
     with open(log, "w") as f:
+        for src, obj, cmd, r in results:
+            f.write(" ".join(cmd) + "\n" + r.stdout + r.stderr)
+    bad = [r for r in results if r[3].returncode != 0]
+    if bad:
+        sys.stderr.write(bad[0][3].stderr[-4000:])
+        raise RuntimeError(f"nvcc failed for {[os.path.basename(b[0]) for b in bad]}; see {log}")
+    cmd = [NVCC, *ARCH, "-shared", "-o", LIB + ".tmp", *[r[1] for r in results]]
+    r = subprocess.run(cmd, capture_output=True, text=True)
+    with open(log, "a") as f:
         f.write(" ".join(cmd) + "\n" + r.stdout + r.stderr)
     if r.returncode != 0:
         sys.stderr.write(r.stderr[-4000:])
-        raise RuntimeError(f"nvcc failed ({r.returncode}); see {log}")
+        raise RuntimeError(f"nvcc link failed ({r.returncode}); see {log}")
     os.replace(LIB + ".tmp", LIB)
     if verbose:
-        print(f"built {LIB}")
+        print(f"built {LIB} from {len(srcs)} translation units")
     return LIB
 
 

@@ -21,12 +21,36 @@ enum Mode : uint32_t { MODE_SORT = 0, MODE_PARTITION = 1, MODE_PARTITION_BY = 2 
 struct NoVal {};
 template <class V> constexpr bool kHasVal = !std::is_same<V, NoVal>::value;
 
+// Bit-exact reinterpretation (keys may be floating point).
+template <class T, class U>
+__device__ __forceinline__ T bit_cast_dev(const U& u) {
+  static_assert(sizeof(T) == sizeof(U), "size mismatch");
+  T t;
+  memcpy(&t, &u, sizeof(T));
+  return t;
+}
+
 // Keys are ordered only through a comparator.
 struct Less {
   template <class T> __device__ __forceinline__ bool operator()(const T& a, const T& b) const { return a < b; }
 };
 struct Greater {
   template <class T> __device__ __forceinline__ bool operator()(const T& a, const T& b) const { return b < a; }
+};
+// IEEE-754 total order for floating-point keys: -NaN < -inf < ... < -0 < +0 <
+// ... < +inf < +NaN, i.e. a strict weak (in fact total) order on bit patterns.
+struct TotalLess {
+  __device__ __forceinline__ static uint32_t rank(float x) {
+    const uint32_t b = bit_cast_dev<uint32_t>(x);
+    return b ^ ((b >> 31) ? 0xffffffffu : 0x80000000u);
+  }
+  __device__ __forceinline__ static unsigned long long rank(double x) {
+    const unsigned long long b = bit_cast_dev<unsigned long long>(x);
+    return b ^ ((b >> 63) ? 0xffffffffffffffffull : 0x8000000000000000ull);
+  }
+  template <class T> __device__ __forceinline__ bool operator()(const T& a, const T& b) const {
+    return rank(a) < rank(b);
+  }
 };
 
 // A bucket being split at some level (one row of the paper's k x p table
@@ -196,19 +220,19 @@ template <class T>
 __device__ __forceinline__ void load_pred(T& a, T& b, const T* p, bool pred) {
   const uint32_t s = (uint32_t)__cvta_generic_to_shared(p);
   if constexpr (sizeof(T) == 8) {
-    unsigned long long x = (unsigned long long)a, y = (unsigned long long)b;
+    unsigned long long x = bit_cast_dev<unsigned long long>(a), y = bit_cast_dev<unsigned long long>(b);
     asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.shared.u64 %0, [%3];\n\t"
                  "@!q ld.shared.u64 %1, [%3];\n\t}"
                  : "+l"(x), "+l"(y)
                  : "r"((uint32_t)pred), "r"(s));
-    a = (T)x; b = (T)y;
+    a = bit_cast_dev<T>(x); b = bit_cast_dev<T>(y);
   } else if constexpr (sizeof(T) == 4) {
-    uint32_t x = (uint32_t)a, y = (uint32_t)b;
+    uint32_t x = bit_cast_dev<uint32_t>(a), y = bit_cast_dev<uint32_t>(b);
     asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.shared.u32 %0, [%3];\n\t"
                  "@!q ld.shared.u32 %1, [%3];\n\t}"
                  : "+r"(x), "+r"(y)
                  : "r"((uint32_t)pred), "r"(s));
-    a = (T)x; b = (T)y;
+    a = bit_cast_dev<T>(x); b = bit_cast_dev<T>(y);
   }
 }
 

@@ -155,11 +155,11 @@ __device__ __forceinline__ Key ld_shared(uint32_t a) {
   if constexpr (sizeof(Key) == 8) {
     unsigned long long x;
     asm volatile("ld.shared.u64 %0, [%1];" : "=l"(x) : "r"(a));
-    return (Key)x;
+    return bit_cast_dev<Key>(x);
   } else {
     uint32_t x;
     asm volatile("ld.shared.u32 %0, [%1];" : "=r"(x) : "r"(a));
-    return (Key)x;
+    return bit_cast_dev<Key>(x);
   }
 }
 __device__ __forceinline__ void red_shared_add(uint32_t a, uint32_t v) {

@@ -312,3 +312,55 @@ def test_host_pipeline(gss, width, pairs):
         np.testing.assert_array_equal(hos[i].numpy(), np.sort(xs[i]))
         if pairs:
             check_pairs(xs[i], hvo[i].numpy(), np.sort(xs[i]))
+
+
+# ---------------------------------------------------------------------------
+# Float keys: IEEE-754 totalOrder (gss_sort_f32 / gss_sort_f64)
+# ---------------------------------------------------------------------------
+def _total_order_bits(bits: np.ndarray, width: int) -> np.ndarray:
+    """IEEE 754-2008 5.10 totalOrder as an unsigned integer order: negative
+    numbers (sign bit set) reverse, positives follow them."""
+    top = np.uint64(1) << np.uint64(width - 1)
+    full = np.uint64((1 << width) - 1)
+    b = bits.astype(np.uint64)
+    return np.where(b & top, b ^ full, b | top)
+
+
+def _from_total_order_bits(r: np.ndarray, width: int) -> np.ndarray:
+    top = np.uint64(1) << np.uint64(width - 1)
+    full = np.uint64((1 << width) - 1)
+    return np.where(r & top, r ^ top, r ^ full)
+
+
+@pytest.mark.parametrize("width", [32, 64])
+def test_float_total_order(gss, oracle_mod, width):
+    ft, ut = (np.float32, np.uint32) if width == 32 else (np.float64, np.uint64)
+    n = (1 << 20) + 999
+    rng = np.random.default_rng(width)
+    x = (rng.standard_normal(n) * rng.choice([1e-30, 1.0, 1e20], n)).astype(ft)
+    special = np.array([np.nan, -np.nan, np.inf, -np.inf, 0.0, -0.0, np.finfo(ft).tiny / 4,
+                        -np.finfo(ft).tiny / 4, np.finfo(ft).max, -np.finfo(ft).max], dtype=ft)
+    idx = rng.integers(0, n, 4096)
+    x[idx] = special[rng.integers(0, special.size, idx.size)]
+    x[:1000] = x[1000:2000]                                  # duplicates
+    bits = x.view(ut)
+    ko, _, st = gss.sort(to_dev(x), M=4096, stats=True)
+    assert st.error_flags == 0
+    got = to_host(ko).view(ut)
+    # the oracle sorts the totalOrder images of the same bit patterns
+    ranks = _total_order_bits(bits, width)
+    ok, _, recs = oracle_mod.sort(ranks, None, oracle_params(oracle_mod, M=4096), log=True)
+    want = _from_total_order_bits(ok.astype(np.uint64), width).astype(ut)
+    np.testing.assert_array_equal(got, want)
+    for lvl in range(3):
+        assert st.split_elems[lvl] == sum(r.m for r in recs if r.level == lvl)
+    # independent check on the ordinary numbers: numpy's float order
+    y = to_host(ko)
+    fin = y[np.isfinite(y) & (y != 0)]
+    np.testing.assert_array_equal(fin, np.sort(x[np.isfinite(x) & (x != 0)]))
+    # -NaN first, +NaN last, -0 before +0
+    sgn = np.signbit(y)
+    nan = np.isnan(y)
+    assert np.all(nan[:int((nan & sgn).sum())]) and np.all(nan[n - int((nan & ~sgn).sum()):])
+    z = np.flatnonzero(y == 0)
+    assert np.all(np.diff(sgn[z].astype(np.int8)) <= 0)
