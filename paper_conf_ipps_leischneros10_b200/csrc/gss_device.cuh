@@ -66,7 +66,7 @@ struct Bucket {
   uint32_t hist_base;      // start of this bucket's K x ntiles histogram (bucket-major)
   uint32_t spl_base;       // start of its splitter storage: tree[kb] then sorted spl[kb]
   uint32_t clamp;          // partition_by: ids are min(b, K-1)
-  uint32_t pad;
+  uint32_t id_base;        // start of its stored bucket ids (16-byte aligned; tile t at id_base + t*T)
 };
 
 struct Item {              // a final bucket (small sort / copy / overflow work)
@@ -76,6 +76,7 @@ struct Item {              // a final bucket (small sort / copy / overflow work)
 struct LevelCounters {
   uint32_t num_buckets, num_tiles, hist_alloc, spl_alloc;
   unsigned long long split_elems;
+  uint32_t id_alloc, pad;  // stored bucket ids: each bucket's range rounded up to 16 elements
 };
 
 struct Counters {

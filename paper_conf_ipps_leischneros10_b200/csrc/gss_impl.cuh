@@ -34,6 +34,7 @@ struct gss_profiler {
 namespace gssh {
 
 inline constexpr uint32_t kVersion = 1;
+inline constexpr uint32_t kFlagScatterFast = 1u << 30;   // experimental scatter variant (k_scatter_fast)
 inline constexpr uint32_t kClassCap[kNumClasses] = {512, 1024, 2048, 4096, 8192, 16384};
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
@@ -152,7 +153,7 @@ struct Layout {
     off_cnt = take(sizeof(Counters));
     off_ktmp = take(n * sizeof(Key));
     off_vtmp = kHasVal<Val> ? take(n * sizeof(Val)) : 0;
-    off_ids = take(n * sizeof(IdT));
+    off_ids = take((n + 16 * ((size_t)cap_buckets + 2)) * sizeof(IdT));   // per-bucket 16-aligned id ranges
     for (int s = 0; s < 2; s++) {
       off_bk[s] = take((size_t)cap_buckets * sizeof(Bucket));
       off_tb[s] = take((size_t)cap_tiles * 4);
@@ -316,7 +317,7 @@ struct Engine {
     auto ks = k_sample<Key, Val, IdT, Cmp>;
     const size_t sm_sample = CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
     auto kc = k_classify<Key, Val, IdT, Cmp>;
-    const size_t sm_cls = (size_t)kmax * sizeof(Key) * 2 + (size_t)(kClsThreads / 32) * kmax * 4;
+    const size_t sm_cls = cls_smem_bytes<Key>(kmax);
     auto ksc = k_scatter<Key, Val, IdT, Cmp>;
     const size_t sm_sc = ScatterSmem<Key, Val, IdT>::bytes(kmax);
     GSS_TRY(set_smem(ks, sm_sample));
@@ -327,6 +328,10 @@ struct Engine {
     if (!g_plan) g_plan = grid_for(k_plan<Key, Val, IdT>, kPlanThreads, 0, di.sms);
     const int g_cls = grid_for(kc, kClsThreads, sm_cls, di.sms);
     const int g_sc = grid_for(ksc, kScatterThreads, sm_sc, di.sms);
+    auto ksf = k_scatter_fast<Key, Val, IdT, Cmp>;
+    const size_t sm_sf = ScatterFastSmem<Key, Val, IdT>::bytes(kmax);
+    GSS_TRY(set_smem(ksf, sm_sf));
+    const int g_sf = grid_for(ksf, kScatterThreads, sm_sf, di.sms);
     auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
     const size_t sm_sd = (size_t)kmax * 4;
     GSS_TRY(set_smem(ksd, sm_sd));
@@ -342,8 +347,10 @@ struct Engine {
                      [&] { k_scan_reduce<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
       GSS_TRY(launch(prof, GSS_K_SCAN, s, count,
                      [&] { k_scan_final<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
-      if (!(cfg.flags & GSS_FLAG_DIRECT_SCATTER) || c.stable) {
+      if (c.stable || !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterFast))) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));
+      } else if (cfg.flags & kFlagScatterFast) {
+        GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksf<<<g_sf, kScatterThreads, sm_sf, s>>>(c, l, kmax); }));
       } else {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count,
                        [&] { ksd<<<g_sd, kDirectThreads, sm_sd, s>>>(c, l); }));

@@ -52,7 +52,7 @@ __global__ void k_init(Ctx<Key, Val, IdT> c) {
   uint32_t nt = (c.n + c.T - 1) / c.T;
   Bucket B{};
   B.lo = 0; B.m = c.n; B.tile_start = 0; B.ntiles = nt; B.kb = kb;
-  B.hist_base = 0; B.spl_base = 0;
+  B.hist_base = 0; B.spl_base = 0; B.id_base = 0;
   c.bk[0][0] = B;
   LevelCounters& L = c.cnt->lvl[0];
   L.num_buckets = 1; L.num_tiles = nt; L.hist_alloc = max(kb, 3u) * nt; L.spl_alloc = 2 * kb;
@@ -166,70 +166,201 @@ __device__ __forceinline__ void red_shared_add(uint32_t a, uint32_t v) {
   asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(a), "r"(v));
 }
 
-// U keys per thread in flight; the descent depth log2(k_s) is uniform per
-// tile, so it is a runtime loop around a fully unrolled U-key body.  The
-// tree index j is kept as a shared-memory byte address a = tb + w*j, so each
-// level of Algorithm 2 (j := 2j + (e > bt[j])) is one load, the comparison
-// and a' = 2a - tb + w*[bt[j] < e].
-template <class Key, class IdT, class Cmp>
-__device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* __restrict__ ids, uint32_t beg,
-                                              uint32_t len, uint32_t tree_s, const Key* spl, uint32_t logk,
-                                              uint32_t ks, uint32_t K, bool eq, bool clamp, uint32_t wc_s, Cmp less) {
-  constexpr int U = 8;
+// Tree layout in shared memory.  Levels 0..4 (nodes 1..31) stay in plain
+// Eytzinger order: a warp touches at most 16 distinct nodes of one level, all
+// inside 128 B, so those loads are conflict-free broadcasts.  Levels 5..7
+// (nodes 32..255) are where 32 lanes hit up to 32 different nodes; there every
+// node is replicated once per bank group (128 B per node: 32 copies of a u32
+// key, 16 of a u64 key) and lane l reads copy l mod (128/w), so a warp's load
+// is conflict-free whatever the keys are.  Levels >= 8 (k > 256) fall back to
+// the plain order.
+constexpr uint32_t kTopLevels = 5;
+constexpr uint32_t kRepEnd = 8;
+constexpr uint32_t kRepNodes = (1u << kRepEnd) - (1u << kTopLevels);    // 224
+template <class Key>
+constexpr uint32_t rep_copies() { return 128u / sizeof(Key); }
+template <class Key>
+constexpr size_t cls_smem_bytes(uint32_t kmax) {
+  return (size_t)kmax * sizeof(Key) * 2 + (size_t)kRepNodes * 128 + (size_t)(kClsThreads / 32) * kmax * 4 +
+         (size_t)(kClsThreads / 32) * 256 * 2;
+}
+
+// One level of Algorithm 2 (j := 2j + (e > bt[j])) on a node address
+// a = base + step*j: a' = 2a - base + step*[bt[j] < e]  (the doubling on the
+// FMA pipe, the comparison and select on the ALU pipe).
+template <class Key, class Cmp>
+__device__ __forceinline__ uint32_t descend_step(uint32_t a, Key e, uint32_t s0, uint32_t s1, Cmp less) {
+  const Key x = ld_shared<Key>(a);
+  const uint32_t t = less(x, e) ? s1 : s0;
+  uint32_t r;
+  asm("mad.lo.u32 %0, %1, 2, %2;" : "=r"(r) : "r"(a), "r"(t));
+  return r;
+}
+
+// Bucket ids of U keys per lane: the whole descent (plain top levels,
+// bank-replicated middle levels, plain deep levels), then the id rule of the
+// tile's mode (0: range buckets, 1: equality mode R4, 2: clamped ids of
+// partition_by).
+template <int MODE, int U, class Key, class Cmp>
+__device__ __forceinline__ void descend_group(const Key (&e)[U], uint32_t (&id)[U], uint32_t tree_s, uint32_t rep_b,
+                                              const Key* spl, uint32_t logk, uint32_t ks, uint32_t K, Cmp less) {
   constexpr uint32_t W = sizeof(Key);
-  const uint32_t step0 = 0u - tree_s, step1 = W - tree_s;
-  const Key* sp = src + beg;
-  IdT* ip = ids + beg;
-  for (uint32_t i0 = threadIdx.x; i0 < len; i0 += U * kClsThreads) {
-    Key e[U];
+  const uint32_t r0 = 0u - rep_b, r1 = 128u - rep_b;         // replicated region steps (per lane)
+  const uint32_t d1 = min(logk, kTopLevels), d2 = min(logk, kRepEnd);
+  // plain region: r = W*j relative to the tree, r' = 2r + W*[bt[j] < e]
+  uint32_t r[U];
+#pragma unroll
+  for (int u = 0; u < U; u++) r[u] = W;
+  for (uint32_t d = 0; d < d1; d++) {
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const Key x = ld_shared<Key>(tree_s + r[u]);
+      const uint32_t t = less(x, e[u]) ? W : 0u;
+      asm("mad.lo.u32 %0, %1, 2, %2;" : "=r"(r[u]) : "r"(r[u]), "r"(t));
+    }
+  }
+  if (logk > kTopLevels) {
+    // replicated region: absolute a = rep_b + 128 j
     uint32_t a[U];
 #pragma unroll
-    for (int u = 0; u < U; u++) {
-      const uint32_t i = i0 + u * kClsThreads;
-      a[u] = tree_s + W;
-      if (i < len) e[u] = sp[i];
+    for (int u = 0; u < U; u++) a[u] = rep_b + (128u / W) * r[u];
+    for (uint32_t d = kTopLevels; d < d2; d++) {
+#pragma unroll
+      for (int u = 0; u < U; u++) a[u] = descend_step(a[u], e[u], r0, r1, less);
     }
-    for (uint32_t d = 0; d < logk; d++) {
+#pragma unroll
+    for (int u = 0; u < U; u++) r[u] = (a[u] - rep_b) / (128u / W);
+    for (uint32_t d = kRepEnd; d < logk; d++) {
 #pragma unroll
       for (int u = 0; u < U; u++) {
-        const Key x = ld_shared<Key>(a[u]);
-        a[u] = a[u] + a[u] + (less(x, e[u]) ? step1 : step0);
+        const Key x = ld_shared<Key>(tree_s + r[u]);
+        const uint32_t t = less(x, e[u]) ? W : 0u;
+        asm("mad.lo.u32 %0, %1, 2, %2;" : "=r"(r[u]) : "r"(r[u]), "r"(t));
       }
     }
+  }
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    const uint32_t b = r[u] / W - (1u << logk);
+    if constexpr (MODE == 1) {
+      // equality bucket of splitter b (b < ks-1 and e == spl[b]: ties go left, so e <= spl[b])
+      const uint32_t bb = min(b, ks - 2);
+      id[u] = 2 * b + ((b + 1 < ks && !less(e[u], spl[bb])) ? 1u : 0u);
+    } else if constexpr (MODE == 2) {
+      id[u] = min(b, K - 1);
+    } else {
+      id[u] = b;
+    }
+  }
+}
+
+// Warp-contiguous groups: warp w of the CTA handles keys [g + 256 w, g + 256 w
+// + 256) of each 2048-key group g, lane l the keys 32u + l (coalesced loads);
+// the warp stages its 256 ids in shared memory and writes them as one 8-byte
+// store per lane.  Full groups run without bounds tests; the next group's
+// keys are loaded before this group descends.
+template <int MODE, class Key, class IdT, class Cmp>
+__device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* __restrict__ tids, uint32_t beg,
+                                              uint32_t len, uint32_t tree_s, uint32_t rep_b, const Key* spl,
+                                              uint32_t logk, uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid,
+                                              Cmp less) {
+  constexpr int U = 8;
+  constexpr uint32_t G = U * kClsThreads;                      // keys per group
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  const uint32_t off = (uint32_t)w * (32 * U) + lane;
+  const Key* sp = src + beg + off;
+  const uint32_t nfull = len / G;
+  Key nx[U];
+  if (nfull) {
+#pragma unroll
+    for (int u = 0; u < U; u++) nx[u] = sp[u * 32];
+  }
+  for (uint32_t g = 0; g < nfull; g++) {
+    Key e[U];
+#pragma unroll
+    for (int u = 0; u < U; u++) e[u] = nx[u];
+    if (g + 1 < nfull) {
+#pragma unroll
+      for (int u = 0; u < U; u++) nx[u] = sp[(g + 1) * G + u * 32];
+    }
+    uint32_t id[U];
+    descend_group<MODE>(e, id, tree_s, rep_b, spl, logk, ks, K, less);
 #pragma unroll
     for (int u = 0; u < U; u++) {
-      const uint32_t i = i0 + u * kClsThreads;
+      red_shared_add(wc_s + 4 * id[u], 1u);
+      wid[u * 32 + lane] = (IdT)id[u];
+    }
+    __syncwarp();
+    // lane l writes ids [l*U, l*U + U) of the warp's 256 (U * sizeof(IdT) bytes)
+    IdT* gp = tids + g * G + (uint32_t)w * (32 * U) + lane * U;
+    if constexpr (sizeof(IdT) == 1) {
+      *reinterpret_cast<uint2*>(gp) = *reinterpret_cast<const uint2*>(wid + lane * U);
+    } else {
+      *reinterpret_cast<uint4*>(gp) = *reinterpret_cast<const uint4*>(wid + lane * U);
+    }
+    __syncwarp();
+  }
+  // tail group: bounds-tested
+  const uint32_t tb = nfull * G;
+  if (tb < len) {
+    Key e[U];
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const uint32_t i = tb + off + u * 32;
+      if (i < len) e[u] = src[beg + i];
+      else e[u] = src[beg];
+    }
+    uint32_t id[U];
+    descend_group<MODE>(e, id, tree_s, rep_b, spl, logk, ks, K, less);
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const uint32_t i = tb + off + u * 32;
       if (i < len) {
-        const uint32_t b = (a[u] - tree_s) / W - (1u << logk);
-        uint32_t id = b;
-        if (eq) id = 2 * b + ((b + 1 < ks && !less(e[u], spl[b])) ? 1u : 0u);
-        else if (clamp) id = min(b, K - 1);
-        ip[i] = (IdT)id;
-        red_shared_add(wc_s + 4 * id, 1u);
+        red_shared_add(wc_s + 4 * id[u], 1u);
+        tids[i] = (IdT)id[u];
       }
     }
   }
 }
 
+// Persistent: CTA b classifies the contiguous tile range [b*per, (b+1)*per),
+// so consecutive tiles mostly share a bucket and its tree stays in shared
+// memory.
 template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kClsThreads, 4) k_classify(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+__global__ void __launch_bounds__(kClsThreads, 2) k_classify(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
+  constexpr uint32_t REP = rep_copies<Key>();
   Key* tree = reinterpret_cast<Key*>(smem_raw);
   Key* spl = tree + kmax;
-  uint32_t* wcnt = reinterpret_cast<uint32_t*>(spl + kmax);
+  Key* rep = spl + kmax;                                       // kRepNodes x REP keys
+  uint32_t* wcnt = reinterpret_cast<uint32_t*>(rep + kRepNodes * REP);
   constexpr int NW = kClsThreads / 32;
+  IdT* wid = reinterpret_cast<IdT*>(wcnt + NW * kmax) + (threadIdx.x >> 5) * 256;   // per-warp id staging
   const Cmp less;
   const uint32_t slot = level & 1;
   const uint32_t nt = c.cnt->lvl[level].num_tiles;
   const Key* src = c.keys(c.src(level));
   const int w = threadIdx.x >> 5;
+  const uint32_t per = (nt + gridDim.x - 1) / gridDim.x;
+  const uint32_t t0 = blockIdx.x * per, t1 = min(nt, t0 + per);
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + w * kmax);
+  const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
+  // node j of levels 5..7 is read by this lane at rep_b + 128 j
+  const uint32_t rep_b = (uint32_t)__cvta_generic_to_shared(rep) - (1u << kTopLevels) * 128u +
+                         (threadIdx.x % REP) * (uint32_t)sizeof(Key);
   uint32_t cur = 0xffffffffu;
-  for (uint32_t t = blockIdx.x; t < nt; t += gridDim.x) {
+  for (uint32_t t = t0; t < t1; t++) {
     const uint32_t b = c.tile_bucket[slot][t];
     const Bucket B = c.bk[slot][b];
+    __syncthreads();                                           // previous tile's counters are read
     if (b != cur) {
-      for (uint32_t j = threadIdx.x + 1; j < B.ks; j += kClsThreads) tree[j] = c.spl[slot][B.spl_base + j];
-      for (uint32_t j = threadIdx.x; j + 1 < B.ks; j += kClsThreads) spl[j] = c.spl[slot][B.spl_base + B.kb + j];
+      const Key* g = c.spl[slot] + B.spl_base;
+      for (uint32_t j = threadIdx.x + 1; j < B.ks; j += kClsThreads) tree[j] = g[j];
+      for (uint32_t j = threadIdx.x; j + 1 < B.ks; j += kClsThreads) spl[j] = g[B.kb + j];
+      if (B.ks > (1u << kTopLevels)) {
+        const uint32_t nrep = (min(B.ks, 1u << kRepEnd) - (1u << kTopLevels)) * REP;
+        for (uint32_t q = threadIdx.x; q < nrep; q += kClsThreads) rep[q] = g[(1u << kTopLevels) + q / REP];
+      }
       cur = b;
     }
     for (uint32_t j = threadIdx.x; j < NW * kmax; j += kClsThreads) wcnt[j] = 0;
@@ -237,9 +368,11 @@ __global__ void __launch_bounds__(kClsThreads, 4) k_classify(Ctx<Key, Val, IdT> 
     const uint32_t tl = t - B.tile_start;
     const uint32_t beg = B.lo + tl * c.T;
     const uint32_t len = min(c.T, B.m - tl * c.T);
-    const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + w * kmax);
-    const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
-    classify_tile(src, c.ids, beg, len, tree_s, spl, ilog2(B.ks), B.ks, B.K, B.eq != 0, B.clamp != 0, wc_s, less);
+    const uint32_t logk = ilog2(B.ks);
+    IdT* tids = c.ids + B.id_base + tl * c.T;                  // 16-byte aligned per tile
+    if (B.eq) classify_tile<1>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    else if (B.clamp) classify_tile<2>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    else classify_tile<0>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
     __syncthreads();
     uint32_t* hist = c.hist[slot] + B.hist_base;
     for (uint32_t id = threadIdx.x; id < B.K; id += kClsThreads) {
@@ -248,7 +381,6 @@ __global__ void __launch_bounds__(kClsThreads, 4) k_classify(Ctx<Key, Val, IdT> 
       for (int q = 0; q < NW; q++) s += wcnt[q * kmax + id];
       hist[id * B.ntiles + tl] = s;
     }
-    __syncthreads();
   }
 }
 
@@ -377,6 +509,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
   uint32_t t = blockIdx.x;
   if (t >= nt) return;
   // tile state
+  uint32_t idb = 0;
   auto tile_info = [&](uint32_t tt, uint32_t& beg, uint32_t& len, uint32_t& K, uint32_t& hrow, uint32_t& hstride,
                        uint32_t& tl, uint32_t& lo) {
     const uint32_t b = c.tile_bucket[slot][tt];
@@ -388,6 +521,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
     hrow = B.hist_base;
     hstride = B.ntiles;
     lo = B.lo;
+    idb = B.id_base + tl * c.T;
   };
   uint32_t beg, len, K, hrow, hstride, tl, blo;
   tile_info(t, beg, len, K, hrow, hstride, tl, blo);
@@ -400,20 +534,20 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
   Key pk[kScatterIter];
   Val pv[kScatterIter];
   uint32_t pid[kScatterIter];
-  auto load_chunk = [&](uint32_t cbeg, uint32_t clen) {
+  auto load_chunk = [&](uint32_t cbeg, uint32_t cid, uint32_t clen) {
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
       const uint32_t q = q0 + it * 32;
       pid[it] = 0xffffffffu;
       if (q < clen) {
         pk[it] = ksrc[cbeg + q];
-        pid[it] = idsrc[cbeg + q];
+        pid[it] = idsrc[cid + q];
         if constexpr (kHasVal<Val>) pv[it] = vsrc[cbeg + q];
       }
     }
   };
   uint32_t c0 = 0;
-  load_chunk(beg, min((uint32_t)kChunk, len));
+  load_chunk(beg, idb, min((uint32_t)kChunk, len));
   for (;;) {
     const uint32_t clen = min((uint32_t)kChunk, len - c0);
     Key kk[kScatterIter];
@@ -521,7 +655,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
         new_tile = true;
       }
     }
-    if (!done) load_chunk(beg + c0, min((uint32_t)kChunk, len - c0));
+    if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
     // write this chunk's bucket runs
 #pragma unroll 4
     for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
@@ -535,6 +669,213 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
       const uint32_t* hist = c.hist[slot] + hrow;
       const uint32_t hb = hist[0];
       for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
+    }
+  }
+}
+
+// Phase 4, default variant.  Every key takes its rank within (warp, chunk,
+// id) from one shared-memory atomic on its warp's counters (a warp whose 32
+// keys share an id -- sorted input -- takes one update for all of them), so
+// the result is deterministic though not stable (R7); a thread per id turns
+// the warp counts into warp starts, warp 0 scans the K chunk totals; the
+// chunk is reordered by id in shared memory and each bucket run is written
+// with coalesced stores.  CTA b handles the contiguous tile range [b*per,
+// (b+1)*per); the next chunk's keys, values and ids are loaded into registers
+// before the current chunk's runs are written out.
+template <class Key, class Val, class IdT>
+struct ScatterFastSmem {
+  static size_t bytes(uint32_t kmax) {
+    size_t b = (size_t)kmax * 4 * 4;                            // ctot, off, delta, gbase
+    b += (size_t)(kScatterThreads / 32) * kmax * 4;             // per-warp counters
+    b = (b + 15) & ~size_t(15);
+    b += (size_t)kChunk * sizeof(Key);
+    if (kHasVal<Val>) b += (size_t)kChunk * sizeof(Val);
+    b += (size_t)kChunk * sizeof(IdT);
+    return b;
+  }
+};
+
+template <class Key, class Val, class IdT, class Cmp>
+__global__ void __launch_bounds__(kScatterThreads, 2)
+    k_scatter_fast(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  constexpr int NW = kScatterThreads / 32;
+  uint32_t* ctot = reinterpret_cast<uint32_t*>(smem_raw);
+  uint32_t* off = ctot + kmax;
+  uint32_t* delta = off + kmax;
+  uint32_t* gbase = delta + kmax;
+  uint32_t* wcnt = gbase + kmax;                                   // NW x kmax
+  size_t o = ((size_t)kmax * 16 + (size_t)NW * kmax * 4 + 15) & ~size_t(15);
+  Key* skeys = reinterpret_cast<Key*>(smem_raw + o);
+  o += (size_t)kChunk * sizeof(Key);
+  Val* svals = reinterpret_cast<Val*>(smem_raw + o);
+  if constexpr (kHasVal<Val>) o += (size_t)kChunk * sizeof(Val);
+  IdT* sids = reinterpret_cast<IdT*>(smem_raw + o);
+
+  const uint32_t slot = level & 1;
+  const uint32_t nt = c.cnt->lvl[level].num_tiles;
+  const uint32_t sb = c.src(level), db = c.dst(level);
+  const Key* ksrc = c.keys(sb);
+  Key* kdst = c.wkeys(db);
+  const Val* vsrc = nullptr;
+  Val* vdst = nullptr;
+  if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
+  const IdT* idsrc = c.ids;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  uint32_t* wc = wcnt + w * kmax;
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
+  const uint32_t q0 = w * (32 * kScatterIter) + lane;
+  const uint32_t per = (nt + gridDim.x - 1) / gridDim.x;
+  uint32_t t = blockIdx.x * per;
+  const uint32_t t_end = min(nt, t + per);
+  if (t >= t_end) return;
+
+  uint32_t beg, len, K, hrow, hstride, tl, blo, idb;
+  auto tile_info = [&](uint32_t tt) {
+    const uint32_t b = c.tile_bucket[slot][tt];
+    const Bucket B = c.bk[slot][b];
+    tl = tt - B.tile_start;
+    beg = B.lo + tl * c.T;
+    len = min(c.T, B.m - tl * c.T);
+    K = B.K;
+    hrow = B.hist_base;
+    hstride = B.ntiles;
+    blo = B.lo;
+    idb = B.id_base + tl * c.T;
+  };
+  auto load_gbase = [&]() {
+    const uint32_t* hist = c.hist[slot] + hrow;
+    const uint32_t hb = hist[0];
+    for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
+  };
+  tile_info(t);
+  load_gbase();
+  Key pk[kScatterIter];
+  Val pv[kScatterIter];
+  uint32_t pid[kScatterIter];
+  auto load_chunk = [&](uint32_t cbeg, uint32_t cid, uint32_t clen) {
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      const uint32_t q = q0 + it * 32;
+      pid[it] = 0xffffffffu;
+      if (q < clen) {
+        pk[it] = ksrc[cbeg + q];
+        pid[it] = idsrc[cid + q];
+        if constexpr (kHasVal<Val>) pv[it] = vsrc[cbeg + q];
+      }
+    }
+  };
+  uint32_t c0 = 0;
+  load_chunk(beg, idb, min((uint32_t)kChunk, len));
+  __syncthreads();                                                 // gbase initialised
+  for (;;) {
+    const uint32_t clen = min((uint32_t)kChunk, len - c0);
+    Key kk[kScatterIter];
+    Val vv[kScatterIter];
+    uint32_t iid[kScatterIter], rk[kScatterIter];
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      kk[it] = pk[it];
+      iid[it] = pid[it];
+      if constexpr (kHasVal<Val>) vv[it] = pv[it];
+    }
+    // 1. ranks within (warp, id), from the warp's own counters: deterministic
+    //    (one warp's atomics are applied in a fixed order)
+    for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
+    __syncwarp();
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      const uint32_t id = iid[it];
+      const uint32_t first = __shfl_sync(kFull, id, 0);
+      if (__all_sync(kFull, id == first) && first != 0xffffffffu) {
+        uint32_t base = 0;
+        if (lane == 0) { base = wc[first]; wc[first] = base + 32u; }
+        __syncwarp();
+        rk[it] = __shfl_sync(kFull, base, 0) + (uint32_t)lane;
+      } else {
+        rk[it] = atom_add_shared_if(id != 0xffffffffu ? 1u : 0u, wc_s + 4 * (id & 0xffffu), 1u);
+      }
+    }
+    __syncthreads();
+    // 2. per id: chunk total and every warp's start within the id's run
+    for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) {
+      uint32_t run = 0;
+#pragma unroll
+      for (int q = 0; q < NW; q++) {
+        const uint32_t x = wcnt[q * kmax + id];
+        wcnt[q * kmax + id] = run;
+        run += x;
+      }
+      ctot[id] = run;
+    }
+    __syncthreads();
+    // 3. warp 0: exclusive scan of the K chunk totals; staged position of id's
+    //    run (off) and staged -> global displacement (delta)
+    if (w == 0) {
+      uint32_t run = 0;
+      for (uint32_t id0 = 0; id0 < K; id0 += 32 * 8) {
+        const uint32_t ib = id0 + lane * 8;
+        uint32_t x[8], sum = 0;
+#pragma unroll
+        for (int j = 0; j < 8; j++) {
+          x[j] = ib + j < K ? ctot[ib + j] : 0u;
+          sum += x[j];
+        }
+        uint32_t inc = sum;
+#pragma unroll
+        for (int sh = 1; sh < 32; sh <<= 1) {
+          const uint32_t y = __shfl_up_sync(kFull, inc, sh);
+          if (lane >= sh) inc += y;
+        }
+        uint32_t ex = run + inc - sum;
+#pragma unroll
+        for (int j = 0; j < 8; j++) {
+          if (ib + j < K) {
+            off[ib + j] = ex;
+            delta[ib + j] = gbase[ib + j] - ex;
+            gbase[ib + j] += x[j];
+          }
+          ex += x[j];
+        }
+        run += __shfl_sync(kFull, inc, 31);
+      }
+    }
+    __syncthreads();
+    // 3. reorder the chunk by id in shared memory
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      if (iid[it] != 0xffffffffu) {
+        const uint32_t pos = off[iid[it]] + wc[iid[it]] + rk[it];
+        skeys[pos] = kk[it];
+        if constexpr (kHasVal<Val>) svals[pos] = vv[it];
+        sids[pos] = (IdT)iid[it];
+      }
+    }
+    // advance and prefetch the next chunk (possibly of the next tile)
+    const uint32_t cur_clen = clen;
+    bool new_tile = false, done = false;
+    c0 += kChunk;
+    if (c0 >= len) {
+      t++;
+      c0 = 0;
+      if (t >= t_end) done = true;
+      else { tile_info(t); new_tile = true; }
+    }
+    if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
+    __syncthreads();
+    // 4. write this chunk's bucket runs
+#pragma unroll 4
+    for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
+      const uint32_t d = delta[sids[q]] + q;
+      kdst[d] = skeys[q];
+      if constexpr (kHasVal<Val>) vdst[d] = svals[q];
+    }
+    if (done) break;
+    if (new_tile) {
+      // gbase is rewritten only after every thread has left step 4
+      __syncthreads();
+      load_gbase();
+      __syncthreads();
     }
   }
 }
@@ -574,7 +915,7 @@ __global__ void __launch_bounds__(kDirectThreads, 4) k_scatter_direct(Ctx<Key, V
     for (uint32_t id = threadIdx.x; id < B.K; id += kDirectThreads) cursor[id] = hist[id * B.ntiles + tl] - hb + B.lo;
     __syncthreads();
     const Key* ks = ksrc + beg;
-    const IdT* is = c.ids + beg;
+    const IdT* is = c.ids + B.id_base + tl * c.T;
     const Val* vs = nullptr;
     if constexpr (kHasVal<Val>) vs = vsrc + beg;
     for (uint32_t w0 = threadIdx.x & ~31u; w0 < len; w0 += U * kDirectThreads) {   // warp-uniform trip count
@@ -722,6 +1063,7 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
         const uint32_t ts = warp_append(&NL.num_tiles, nt);
         const uint32_t hbn = warp_append(&NL.hist_alloc, to_next ? max(kb, 3u) * nt : 0u);
         const uint32_t sbn = warp_append(&NL.spl_alloc, 2 * kb);
+        const uint32_t ib = warp_append(&NL.id_alloc, to_next ? (m + 15u) & ~15u : 0u);
         const uint64_t el = warp_sum64(to_next ? m : 0);
         if (lane == 0 && el) atomicAdd(&NL.split_elems, (unsigned long long)el);
         if (to_next) {
@@ -730,6 +1072,7 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
             Bucket nbk{};
             nbk.lo = start; nbk.m = m; nbk.tile_start = ts; nbk.ntiles = nt; nbk.kb = kb;
             nbk.hist_base = hbn; nbk.spl_base = sbn;
+            nbk.id_base = ib;                                     // 16-element aligned, disjoint per bucket
             c.bk[next & 1][bi] = nbk;
           } else {
             atomicOr(&c.cnt->err, 4u);
