@@ -294,65 +294,126 @@ constexpr int sort_items() {
   return (kHasVal<Val> && sizeof(Key) + sizeof(Val) > 8) ? 8 : 16;
 }
 
+// Runs of every round are stored so that each merge pair reads as one
+// bitonic sequence: run r is kept ascending when r is even and descending when
+// r is odd.  A merge then walks A upwards from its left end and B downwards
+// from the right end of the pair, and reading past the end of either run
+// lands on a key that can never be taken wrongly:
+//  * past A's end lies B's largest key (B is stored descending right after A);
+//  * past B's smallest key lies A's largest key.
+// Keys only: A is taken iff a < b (B wins ties), so an exhausted A (its
+// "next" is max B >= every b) is never taken, and an exhausted B's stand-in
+// (an A key >= the current a) is taken only when it equals the
+// current a -- the same key value.  With values the stand-ins must never be
+// taken: A wins ties (B's stand-in is >= a, so A is taken) and A carries one
+// index test.  Either way the merge loop has no per-step bounds tests.
 template <class Key, class Val, int NT, class Cmp, int ITEMS_ = sort_items<Key, Val>()>
 struct CtaSort {
   static constexpr int ITEMS = ITEMS_;
   static constexpr int C = NT * ITEMS;
   static constexpr int PL = padded_len(C);
+  static constexpr bool KV = kHasVal<Val>;
+  // keys-only unsigned keys under operator<: the merge step in PTX
+  static constexpr bool kFastMerge = !KV && std::is_same<Cmp, Less>::value && std::is_unsigned<Key>::value &&
+                                     (sizeof(Key) == 4 || sizeof(Key) == 8);
+  __device__ static __forceinline__ void fast_step(Key& out, Key& ka, Key& kb, int& xa, int& xb, uint32_t sb) {
+    if constexpr (sizeof(Key) == 8) {
+      unsigned long long o, a = ka, b = kb;
+      asm volatile(
+          "{\n\t.reg .pred p;\n\t.reg .u32 x, t;\n\t"
+          "setp.ge.u64 p, %1, %2;\n\t"
+          "selp.b64 %0, %2, %1, p;\n\t"
+          "@!p add.s32 %3, %3, 1;\n\t"
+          "@p add.s32 %4, %4, -1;\n\t"
+          "selp.b32 x, %4, %3, p;\n\t"
+          "shr.s32 t, x, 4;\n\t"
+          "add.s32 t, t, x;\n\t"
+          "mad.lo.u32 t, t, 8, %5;\n\t"
+          "@!p ld.volatile.shared.u64 %1, [t];\n\t"
+          "@p ld.volatile.shared.u64 %2, [t];\n\t}"
+          : "=l"(o), "+l"(a), "+l"(b), "+r"(xa), "+r"(xb)
+          : "r"(sb));
+      out = (Key)o; ka = (Key)a; kb = (Key)b;
+    } else {
+      uint32_t o, a = ka, b = kb;
+      asm volatile(
+          "{\n\t.reg .pred p;\n\t.reg .u32 x, t;\n\t"
+          "setp.ge.u32 p, %1, %2;\n\t"
+          "selp.b32 %0, %2, %1, p;\n\t"
+          "@!p add.s32 %3, %3, 1;\n\t"
+          "@p add.s32 %4, %4, -1;\n\t"
+          "selp.b32 x, %4, %3, p;\n\t"
+          "shr.s32 t, x, 4;\n\t"
+          "add.s32 t, t, x;\n\t"
+          "mad.lo.u32 t, t, 4, %5;\n\t"
+          "@!p ld.volatile.shared.u32 %1, [t];\n\t"
+          "@p ld.volatile.shared.u32 %2, [t];\n\t}"
+          : "=r"(o), "+r"(a), "+r"(b), "+r"(xa), "+r"(xb)
+          : "r"(sb));
+      out = (Key)o; ka = (Key)a; kb = (Key)b;
+    }
+  }
   static constexpr size_t smem_bytes() {
     return (size_t)PL * sizeof(Key) + (kHasVal<Val> ? (size_t)PL * sizeof(Val) : 0);
   }
 
-  // Merge-path split of output diagonal `diag` of runs A = sk[a0, a0+aLen),
-  // B = sk[b0, b0+bLen) (stable: A first on ties), then ITEMS outputs into
-  // k/v.  One branch-free path: a run that is exhausted is never taken, and
-  // the element read one past its end lies inside the buffer and is unused.
-  __device__ static __forceinline__ void merge_items(const Key* sk, const Val* sv, int a0, int aLen, int b0,
-                                                     int bLen, int diag, Key* k, Val* v, Cmp less) {
-    int lo = max(0, diag - bLen), hi = min(diag, aLen);
-    while (lo < hi) {
-      const int mid = (lo + hi) >> 1;
-      if (less(sk[phys(b0 + diag - 1 - mid)], sk[phys(a0 + mid)])) hi = mid; else lo = mid + 1;
+  // ITEMS outputs of the merge of pair (A = run at ps of aLen keys, B = run at
+  // ps + aLen of bLen keys, stored descending), starting at output diag.
+  __device__ static __forceinline__ void merge_items(const Key* sk, const Val* sv, int ps, int aLen, int bLen,
+                                                     int diag, Key* k, Val* v, Cmp less) {
+    const int bEnd = ps + aLen + bLen - 1;                   // B's smallest key
+    int ia;
+    if constexpr (KV) {
+      // number of A keys among the first diag outputs, A first on ties
+      int lo = max(0, diag - bLen), hi = min(diag, aLen);
+      while (lo < hi) {
+        const int mid = (lo + hi) >> 1;
+        if (less(sk[phys(bEnd - (diag - 1 - mid))], sk[phys(ps + mid)])) hi = mid; else lo = mid + 1;
+      }
+      ia = lo;
+    } else {
+      // number of B keys among the first diag outputs, B first on ties
+      int lo = max(0, diag - aLen), hi = min(diag, bLen);
+      while (lo < hi) {
+        const int mid = (lo + hi) >> 1;
+        if (less(sk[phys(ps + diag - 1 - mid)], sk[phys(bEnd - mid)])) hi = mid; else lo = mid + 1;
+      }
+      ia = diag - lo;
     }
-    int ia = a0 + lo, ib = b0 + diag - lo;
-    const int ae = a0 + aLen, be = b0 + bLen;
-    Key ka = sk[phys(ia)], kb = sk[phys(ib)];
-    Val va, vb;
-    if constexpr (kHasVal<Val>) { va = sv[phys(ia)]; vb = sv[phys(ib)]; }
-    if (__all_sync(__activemask(), ia + ITEMS <= ae && ib + ITEMS <= be)) {
-      // no lane can exhaust a run in its window: no bounds tests, and the next
-      // key is loaded straight into the register of the side that advanced
+    int xa = ps + ia, xb = bEnd - (diag - ia);
+    const int ae = ps + aLen;
+    Key ka = sk[phys(xa)], kb = sk[phys(xb)];
+    if constexpr (kFastMerge) {
+      // one compare, the output select, the index step and a predicated load
+      // straight into the consumed head per output
+      const uint32_t sb = (uint32_t)__cvta_generic_to_shared(sk);
 #pragma unroll
       for (int i = 0; i < ITEMS; i++) {
-        const bool p = !less(kb, ka);
-        k[i] = p ? ka : kb;
-        if constexpr (kHasVal<Val>) v[i] = p ? va : vb;
-        if (i + 1 < ITEMS) {
-          const int nx = (p ? ia : ib) + 1;
-          ia = p ? nx : ia;
-          ib = p ? ib : nx;
-          load_pred(ka, kb, sk + phys(nx), p);
-          if constexpr (kHasVal<Val>) load_pred(va, vb, sv + phys(nx), p);
-        }
+        if (i + 1 < ITEMS) fast_step(k[i], ka, kb, xa, xb, sb);
+        else k[i] = ka < kb ? ka : kb;
       }
       return;
     }
+    Val va, vb;
+    if constexpr (KV) { va = sv[phys(xa)]; vb = sv[phys(xb)]; }
 #pragma unroll
     for (int i = 0; i < ITEMS; i++) {
-      const bool p = (ib >= be) || (ia < ae && !less(kb, ka));
+      bool p;
+      if constexpr (KV) p = (xa < ae) && !less(kb, ka);
+      else p = less(ka, kb);
       k[i] = p ? ka : kb;
-      if constexpr (kHasVal<Val>) v[i] = p ? va : vb;
+      if constexpr (KV) v[i] = p ? va : vb;
       if (i + 1 < ITEMS) {
-        const int nx = (p ? ia : ib) + 1;
-        const Key x = sk[phys(nx)];
-        ia = p ? nx : ia;
-        ib = p ? ib : nx;
-        ka = p ? x : ka;
-        kb = p ? kb : x;
-        if constexpr (kHasVal<Val>) {
-          const Val y = sv[phys(nx)];
-          va = p ? y : va;
-          vb = p ? vb : y;
+        const int nx = p ? xa + 1 : xb - 1;
+        xa = p ? nx : xa;
+        xb = p ? xb : nx;
+        const Key y = sk[phys(nx)];
+        ka = p ? y : ka;
+        kb = p ? kb : y;
+        if constexpr (KV) {
+          const Val z = sv[phys(nx)];
+          va = p ? z : va;
+          vb = p ? vb : z;
         }
       }
     }
@@ -361,6 +422,38 @@ struct CtaSort {
   // NT == 32: a single warp sorts on its own (only warp barriers).
   __device__ static __forceinline__ void bar() {
     if constexpr (NT == 32) __syncwarp(); else __syncthreads();
+  }
+
+  // cnt items of a run [rs, rs + rlen) starting at run offset o, ascending or descending
+  __device__ static __forceinline__ void store_run(Key* sk, Val* sv, const Key* k, const Val* v, int cnt, int rs,
+                                                   int rlen, int o, bool desc) {
+    if (ITEMS == 16 && cnt == ITEMS && ((rs + o) & 15) == 0 && (rlen & 15) == 0) {
+      // the ITEMS slots are one padded row: consecutive addresses, immediate offsets
+      if (desc) {
+        const int q = phys(rs + rlen - 1 - o);
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          sk[q - i] = k[i];
+          if constexpr (KV) sv[q - i] = v[i];
+        }
+      } else {
+        const int q = phys(rs + o);
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          sk[q + i] = k[i];
+          if constexpr (KV) sv[q + i] = v[i];
+        }
+      }
+      return;
+    }
+#pragma unroll
+    for (int i = 0; i < ITEMS; i++) {
+      if (i < cnt) {
+        const int q = desc ? rs + rlen - 1 - (o + i) : rs + o + i;
+        sk[phys(q)] = k[i];
+        if constexpr (KV) sv[phys(q)] = v[i];
+      }
+    }
   }
 
   // Sorts sk[phys(0..m)) (and sv) in place; 0 <= m <= C.  Every thread of
@@ -378,7 +471,7 @@ struct CtaSort {
       for (int i = 0; i < ITEMS; i++) {
         if (i < cnt) {
           k[i] = sk[phys(base + i)];
-          if constexpr (kHasVal<Val>) v[i] = sv[phys(base + i)];
+          if constexpr (KV) v[i] = sv[phys(base + i)];
         }
       }
       // A partial thread pads with copies of its largest item: after sorting,
@@ -393,7 +486,7 @@ struct CtaSort {
 #pragma unroll
         for (int i = 1; i < ITEMS; i++)
           if (i < cnt && less(mx, k[i])) { mx = k[i]; vmx = v[i]; }
-        if constexpr (kHasVal<Val>) {
+        if constexpr (KV) {
           int reps = 0;
 #pragma unroll
           for (int i = 0; i < ITEMS; i++)
@@ -408,43 +501,38 @@ struct CtaSort {
           }
         }
       }
-      if constexpr (kHasVal<Val>) {
+      if constexpr (KV) {
         if (stable_path) transposition_sort<ITEMS>(k, v, less);
         else oem_sort<0, ITEMS>(k, v, less);
       } else {
         oem_sort<0, ITEMS>(k, v, less);
       }
-#pragma unroll
-      for (int i = 0; i < ITEMS; i++) {
-        if (i < cnt) {
-          sk[phys(base + i)] = k[i];
-          if constexpr (kHasVal<Val>) sv[phys(base + i)] = v[i];
-        }
-      }
     }
     __syncwarp();
+    if (cnt > 0) store_run(sk, sv, k, v, cnt, base, cnt, 0, (t & 1) != 0);   // run t: descending if t is odd
     // Rounds whose merged pairs (2w keys) lie inside one warp's 32*ITEMS keys
     // only synchronise the warp; wider rounds synchronise the block.
     for (int w = ITEMS; w < m; w *= 2) {
       const bool blk = NT > 32 && 2 * w > 32 * ITEMS;
-      if (blk) __syncthreads();
-      if (cnt > 0) {
-        const int ps = (base / (2 * w)) * (2 * w);
-        const int aLen = min(w, m - ps);
-        const int bLen = max(0, min(w, m - ps - w));
-        merge_items(sk, sv, ps, aLen, ps + w, bLen, base - ps, k, v, less);
-      }
       if (blk) __syncthreads(); else __syncwarp();
+      const int ps = (base / (2 * w)) * (2 * w);
+      const int aLen = min(w, m - ps);
+      const int bLen = max(0, min(w, m - ps - w));
       if (cnt > 0) {
+        if (bLen > 0) {
+          merge_items(sk, sv, ps, aLen, bLen, base - ps, k, v, less);
+        } else {
 #pragma unroll
-        for (int i = 0; i < ITEMS; i++) {
-          if (i < cnt) {
-            sk[phys(base + i)] = k[i];
-            if constexpr (kHasVal<Val>) sv[phys(base + i)] = v[i];
+          for (int i = 0; i < ITEMS; i++) {               // a lone last run: already in place and ascending
+            if (i < cnt) {
+              k[i] = sk[phys(base + i)];
+              if constexpr (KV) v[i] = sv[phys(base + i)];
+            }
           }
         }
       }
-      if (!blk) __syncwarp();
+      if (blk) __syncthreads(); else __syncwarp();
+      if (cnt > 0) store_run(sk, sv, k, v, cnt, ps, aLen + bLen, base - ps, ((base / (2 * w)) & 1) != 0);
     }
     bar();
   }

@@ -19,10 +19,12 @@ raw = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv", "--metrics", "
 tmp = tempfile.mkdtemp()
 if lib.endswith(".so"):
     subprocess.run(["cuobjdump", "-xelf", "all", os.path.abspath(lib)], cwd=tmp, capture_output=True)
-    cub = [os.path.join(tmp, f) for f in os.listdir(tmp) if f.endswith(".cubin")][0]
+    cubs = [os.path.join(tmp, f) for f in sorted(os.listdir(tmp)) if f.endswith(".cubin")]
 else:
-    cub = lib
-sass = subprocess.run(["nvdisasm", "-g", "-c", cub], capture_output=True, text=True).stdout.splitlines()
+    cubs = [lib]
+sass = []
+for cub in cubs:   # libgss.so holds one cubin per translation unit
+    sass += subprocess.run(["nvdisasm", "-g", "-c", cub], capture_output=True, text=True).stdout.splitlines()
 # split functions
 funcs = {}
 cur = None

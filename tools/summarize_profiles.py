@@ -19,6 +19,10 @@ METRICS = {
     "branch_targets": ("smsp__sass_branch_targets.sum", 1),
     "branch_targets_divergent": ("smsp__sass_branch_targets_threads_divergent.sum", 1),
     "threads_per_inst": ("smsp__thread_inst_executed_per_inst_executed.ratio", 1),
+    "pipe_alu_pct": ("sm__inst_executed_pipe_alu.avg.pct_of_peak_sustained_active", 1),
+    "pipe_fma_pct": ("sm__inst_executed_pipe_fma.avg.pct_of_peak_sustained_active", 1),
+    "pipe_lsu_pct": ("sm__inst_executed_pipe_lsu.avg.pct_of_peak_sustained_active", 1),
+    "smem_pipe_pct": ("l1tex__data_pipe_lsu_wavefronts_mem_shared.avg.pct_of_peak_sustained_elapsed", 1),
     "registers": ("launch__registers_per_thread", 1),
     "block": ("launch__block_size", 1),
     "grid": ("launch__grid_size", 1),
@@ -69,7 +73,7 @@ with open(os.path.join(odir, f"{tag}_ncu_summary.md"), "w") as f:
         f.write(f"## {k}\n\n`{e['kernel']}`\n\n")
         for name in ("duration_ms", "dram_read_GB", "dram_write_GB", "dram_GBps", "dram_throughput_pct",
                      "issue_active_pct", "warps_active_pct", "inst_executed", "smem_wavefronts",
-                     "smem_ld_bank_conflicts", "smem_st_bank_conflicts", "divergent_branch_pct",
+                     "smem_ld_bank_conflicts", "smem_st_bank_conflicts", "divergent_branch_pct", "pipe_alu_pct", "pipe_fma_pct", "pipe_lsu_pct", "smem_pipe_pct",
                      "threads_per_inst", "registers", "block", "grid"):
             if name in e:
                 v = e[name]
