@@ -114,8 +114,11 @@ typedef struct gss_params {
                                       CUDA graph on first use and replay it on later calls
                                       with identical buffers, n and parameters (launch-bound
                                       sizes); ignored with stats or a profiler              */
-#define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets with one more sample-sort split inside
-                                      shared memory + warp merge sorts (P:332-335 variant)  */
+#define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets of two or more warps with one more
+                                      sample-sort split inside the SM + warp merge sorts of
+                                      packed segments; ablation: on B200 its
+                                      serial sample/segment phases and partial warps cost
+                                      more than the CTA-wide merge rounds they remove       */
 
 /* Human-readable name of a status code (static storage). */
 const char* gss_status_string(gss_status s);

@@ -20,7 +20,7 @@ LIB = os.path.join(PKG, "libgss.so")
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 FLAGS = ARCH + ["-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr", "-Xcompiler", "-fPIC",
-                "-Xptxas", "-v"]
+                "-Xptxas", "-v"] + os.environ.get("GSS_NVCC_EXTRA", "").split()   # tuning experiments (-D...)
 
 
 def sources():

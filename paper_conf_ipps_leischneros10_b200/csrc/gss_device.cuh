@@ -11,7 +11,13 @@
 
 namespace gss {
 
-constexpr int kNumClasses = 6;        // in-SM sort size classes (512 .. 16K keys)
+// In-SM sort size classes (R8): class i holds buckets sorted by a CTA of
+// class_warps(i) warps, i.e. up to class_warps(i) * 32 * sort_items keys
+// (1..16 warps one by one, then 20, 24, 28, 32).  Fine classes keep every
+// thread of a bucket's CTA busy: with power-of-two classes a bucket just
+// above a class boundary left half of its CTA idle at every merge barrier.
+constexpr int kNumClasses = 20;
+__host__ __device__ constexpr int class_warps(int i) { return i < 16 ? i + 1 : 16 + 4 * (i - 15); }
 constexpr int kMaxLevels = 16;        // distribution levels launched at most
 constexpr uint32_t kFull = 0xffffffffu;
 
@@ -82,8 +88,7 @@ struct LevelCounters {
 struct Counters {
   LevelCounters lvl[kMaxLevels + 1];
   uint32_t small_count[kNumClasses];
-  uint32_t retry_count[kNumClasses];   // sub-buckets the in-SM sample split could not finish
-  uint32_t copy_count, ovf_count, err, pad;
+  uint32_t copy_count, ovf_count, err, fb_count;   // fb: buckets the in-SM split hands to the block sort
   unsigned long long small_elems, max_small, eq_buckets, eq_elems, ovf_elems;
 };
 
@@ -99,14 +104,14 @@ struct Ctx {
   uint32_t* hist[2];
   Key* spl[2];
   Item* small[kNumClasses];
-  Item* retry[kNumClasses];
   Item* copy;
   Item* ovf;
+  Item* fb;
   uint32_t* scan_part;
   const Key* given_spl;              // MODE_PARTITION_BY
   uint32_t given_nspl;
   uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
-  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf;
+  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb;
   uint32_t cap_small[kNumClasses];
   uint32_t class_cap[kNumClasses];
   uint64_t seed;
@@ -419,16 +424,17 @@ struct CtaSort {
     }
   }
 
-  // NT == 32: a single warp sorts on its own (only warp barriers).
-  __device__ static __forceinline__ void bar() {
-    if constexpr (NT == 32) __syncwarp(); else __syncthreads();
+  // A single warp (NT == 32, or a 32-thread block) sorts on its own: only warp barriers.
+  __device__ static __forceinline__ void bar(int nt) {
+    if (NT == 32 || nt == 32) __syncwarp(); else __syncthreads();
   }
 
   // cnt items of a run [rs, rs + rlen) starting at run offset o, ascending or descending
   __device__ static __forceinline__ void store_run(Key* sk, Val* sv, const Key* k, const Val* v, int cnt, int rs,
                                                    int rlen, int o, bool desc) {
-    if (ITEMS == 16 && cnt == ITEMS && ((rs + o) & 15) == 0 && (rlen & 15) == 0) {
-      // the ITEMS slots are one padded row: consecutive addresses, immediate offsets
+    // ascending: slots rs+o .. rs+o+ITEMS-1; descending: rs+rlen-o-ITEMS .. rs+rlen-o-1
+    if (ITEMS <= 16 && cnt == ITEMS && (((desc ? rs + rlen - o : rs + o)) & (ITEMS - 1)) == 0) {
+      // the ITEMS slots lie in one padded row of 16: consecutive addresses, immediate offsets
       if (desc) {
         const int q = phys(rs + rlen - 1 - o);
 #pragma unroll
@@ -456,11 +462,12 @@ struct CtaSort {
     }
   }
 
-  // Sorts sk[phys(0..m)) (and sv) in place; 0 <= m <= C.  Every thread of
-  // the NT-thread block (or every lane of the warp when NT == 32) must call
-  // it.  Begins and ends with a barrier.
-  __device__ static void sort(Key* sk, Val* sv, int m, Cmp less) {
-    bar();
+  // Sorts sk[phys(0..m)) (and sv) in place; 0 <= m <= nt * ITEMS.  Every
+  // thread of the nt-thread block (nt <= NT; nt = NT unless the caller sizes
+  // the block at run time), or every lane of the warp when NT == 32, must
+  // call it.  Begins and ends with a barrier.
+  __device__ static void sort(Key* sk, Val* sv, int m, Cmp less, int nt = NT) {
+    bar(nt);
     const int t = NT == 32 ? (threadIdx.x & 31) : threadIdx.x;
     const int base = t * ITEMS;
     const int cnt = min(max(m - base, 0), ITEMS);
@@ -513,9 +520,9 @@ struct CtaSort {
     // Rounds whose merged pairs (2w keys) lie inside one warp's 32*ITEMS keys
     // only synchronise the warp; wider rounds synchronise the block.
     for (int w = ITEMS; w < m; w *= 2) {
-      const bool blk = NT > 32 && 2 * w > 32 * ITEMS;
+      const bool blk = NT > 32 && nt > 32 && 2 * w > 32 * ITEMS;
       if (blk) __syncthreads(); else __syncwarp();
-      const int ps = (base / (2 * w)) * (2 * w);
+      const int ps = base & ~(2 * w - 1);                // w is a power of two
       const int aLen = min(w, m - ps);
       const int bLen = max(0, min(w, m - ps - w));
       if (cnt > 0) {
@@ -532,9 +539,9 @@ struct CtaSort {
         }
       }
       if (blk) __syncthreads(); else __syncwarp();
-      if (cnt > 0) store_run(sk, sv, k, v, cnt, ps, aLen + bLen, base - ps, ((base / (2 * w)) & 1) != 0);
+      if (cnt > 0) store_run(sk, sv, k, v, cnt, ps, aLen + bLen, base - ps, (base & (2 * w)) != 0);
     }
-    bar();
+    bar(nt);
   }
 };
 

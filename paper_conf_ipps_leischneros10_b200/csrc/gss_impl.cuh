@@ -35,7 +35,6 @@ namespace gssh {
 
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterFast = 1u << 30;   // experimental scatter variant (k_scatter_fast)
-inline constexpr uint32_t kClassCap[kNumClasses] = {512, 1024, 2048, 4096, 8192, 16384};
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -96,10 +95,10 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   c->seed = p.seed ? p.seed : 5489;
   c->flags = p.flags;
   if (c->flags & GSS_FLAG_RECOMPUTE_IDS) return GSS_ERROR_NOT_SUPPORTED;
-  c->nclass = 0;
-  for (int i = 0; i < kNumClasses; i++)
-    if (kClassCap[i] <= cap) c->nclass = i + 1;
-  for (int i = 0; i < kNumClasses; i++) c->class_cap[i] = kClassCap[std::min<int>(i, c->nclass - 1)];
+  // size classes (R8): class i = buckets a CTA of class_warps(i) warps sorts
+  c->nclass = kNumClasses;
+  for (int i = 0; i < kNumClasses; i++) c->class_cap[i] = (uint32_t)(class_warps(i) * 32 * small_items<Key, Val>());
+  if (c->class_cap[kNumClasses - 1] != cap) return GSS_ERROR_NOT_SUPPORTED;
   c->kmax = std::max<uint32_t>(std::max(c->k, kmin_given), 4u);
   // levels: expected depth with children up to 2x the mean, plus one spare level
   if (p.max_levels) {
@@ -121,9 +120,8 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
 template <class Key, class Val, class IdT>
 struct Layout {
   size_t off_cnt, off_ktmp, off_vtmp, off_ids, off_bk[2], off_tb[2], off_hist[2], off_spl[2], off_small[kNumClasses],
-      off_retry[kNumClasses],
-      off_copy, off_ovf, off_scan, off_hin_k, off_hin_v, off_hout_k, off_hout_v, total;
-  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_small[kNumClasses];
+      off_copy, off_ovf, off_fb, off_scan, off_hin_k, off_hin_v, off_hout_k, off_hout_v, total;
+  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb, cap_small[kNumClasses];
 
   void compute(uint64_t n, const Cfg& c, int mode, bool host_io) {
     const uint64_t M = mode == MODE_SORT ? c.M : 0;
@@ -133,12 +131,13 @@ struct Layout {
     cap_spl = 2 * c.kmax * cap_buckets;
     const uint64_t children = (uint64_t)std::max<uint32_t>(c.L, 1) * cap_buckets * std::max(c.kmax, 3u) + 1;
     for (int i = 0; i < kNumClasses; i++) {
-      uint64_t lower = i == 0 ? 0 : kClassCap[i - 1];
+      uint64_t lower = i == 0 ? 0 : c.class_cap[i - 1];
       uint64_t cap = std::min<uint64_t>(children, n / (lower + 1) + 1);
       cap_small[i] = (i < (int)c.nclass) ? (uint32_t)cap : 0;
     }
     cap_copy = (uint32_t)(n / c.T + n / (c.class_cap[kNumClasses - 1] + 1) + 2);
     cap_ovf = cap_buckets;
+    cap_fb = mode == MODE_SORT ? (uint32_t)(n / (c.class_cap[0] + 1) + 1) : 1;   // buckets of the split classes
     size_t o = 0;
     auto take = [&](size_t bytes) { size_t r = o; o = align_up(o + bytes); return r; };
     off_hin_k = off_hout_k = off_hin_v = off_hout_v = 0;
@@ -161,9 +160,9 @@ struct Layout {
       off_spl[s] = take((size_t)cap_spl * sizeof(Key));
     }
     for (int i = 0; i < kNumClasses; i++) off_small[i] = take((size_t)cap_small[i] * sizeof(Item));
-    for (int i = 0; i < kNumClasses; i++) off_retry[i] = take((size_t)cap_small[i] * sizeof(Item));
     off_copy = take((size_t)cap_copy * sizeof(Item));
     off_ovf = take((size_t)cap_ovf * sizeof(Item));
+    off_fb = take((size_t)cap_fb * sizeof(Item));
     off_scan = take(kScanCtas * 4);
     total = o;
   }
@@ -249,12 +248,12 @@ struct Engine {
     }
     for (int i = 0; i < kNumClasses; i++) {
       c.small[i] = reinterpret_cast<Item*>(base + lay.off_small[i]);
-      c.retry[i] = reinterpret_cast<Item*>(base + lay.off_retry[i]);
       c.cap_small[i] = lay.cap_small[i];
       c.class_cap[i] = cfg.class_cap[i];
     }
     c.copy = reinterpret_cast<Item*>(base + lay.off_copy);
     c.ovf = reinterpret_cast<Item*>(base + lay.off_ovf);
+    c.fb = reinterpret_cast<Item*>(base + lay.off_fb);
     c.scan_part = reinterpret_cast<uint32_t*>(base + lay.off_scan);
     c.n = (uint32_t)n;
     c.M = (uint32_t)cfg.M;
@@ -265,47 +264,36 @@ struct Engine {
     c.stable = ((cfg.flags & GSS_FLAG_STABLE) || mode != MODE_SORT) ? 1u : 0u;   // partitions stay stable (R7 probe)
     c.cap_buckets = lay.cap_buckets; c.cap_tiles = lay.cap_tiles; c.cap_hist = lay.cap_hist;
     c.cap_spl = lay.cap_spl; c.cap_copy = lay.cap_copy; c.cap_ovf = lay.cap_ovf;
+    c.cap_fb = lay.cap_fb;
     c.seed = cfg.seed;
     return c;
   }
 
-  template <int CAP>
+  // In-SM sorts of one size class: the block merge sort (k_small_block) by
+  // default; with GSS_FLAG_SPLIT_SORT the sample split + warp segment sorts
+  // (k_small) for classes of two or more warps.  cls == kNumClasses: the
+  // block merge sort of the buckets the split handed back (1024 threads).
   static gss_status launch_small(C& c, const Cfg& cfg, int cls, const DeviceInfo& di, cudaStream_t s,
-                                 gss_profiler* prof, uint32_t* count, uint32_t retry) {
-    constexpr int NT = small_threads<Key, Val, CAP>();
-    auto kern = k_small<Key, Val, IdT, Cmp, CAP>;
-    const size_t smem = CtaSort<Key, Val, NT, Cmp, small_items<Key, Val, CAP>()>::smem_bytes();
-    GSS_TRY(set_smem(kern, smem));
-    static int grid = 0;
-    if (!grid) grid = grid_for(kern, NT, smem, di.sms);
-    return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<grid, NT, smem, s>>>(c, (uint32_t)cls, retry); });
-  }
-
-  template <int CAP>
-  static gss_status launch_split(C& c, const Cfg& cfg, int cls, const DeviceInfo& di, cudaStream_t s,
                                  gss_profiler* prof, uint32_t* count) {
-    constexpr int NT = split_threads<Key, Val, CAP>();
-    auto kern = k_split_sort<Key, Val, IdT, Cmp, CAP>;
-    const size_t smem = SplitSortSmem<Key, Val, CAP, NT>::bytes();
-    GSS_TRY(set_smem(kern, smem));
-    static int grid = 0;
-    if (!grid) grid = grid_for(kern, NT, smem, di.sms);
-    return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<grid, NT, smem, s>>>(c, (uint32_t)cls); });
-  }
-
-  template <int CAP>
-  static gss_status launch_class(C& c, const Cfg& cfg, int cls, const DeviceInfo& di, cudaStream_t s,
-                                 gss_profiler* prof, uint32_t* count, int phase) {
-    // phase 0: the bucket lists; phase 1: the retry lists (sub-buckets an
-    // in-SM split could not finish).  The in-SM sample split (k_split_sort) is
-    // built but not selected: on B200 its warp-level sub-bucket sorts cost more
-    // than the block-wide merge sort (profiles/r01 notes).
-    if (cfg.flags & GSS_FLAG_SPLIT_SORT) {
-      if (phase == 0) return launch_split<CAP>(c, cfg, cls, di, s, prof, count);
-      return launch_small<CAP>(c, cfg, cls, di, s, prof, count, 1u);
+    const bool fb = cls == kNumClasses;
+    const int nt = fb ? kSmallMaxThreads : class_warps(cls) * 32;
+    if (!fb && nt > 32 && (cfg.flags & GSS_FLAG_SPLIT_SORT)) {
+      auto kern = k_small<Key, Val, IdT, Cmp>;
+      const int ns = std::min(nt, kSplitMaxThreads);
+      const size_t smem = small_smem_bytes<Key, Val>(cfg.class_cap[cls]);
+      GSS_TRY(set_smem(kern, small_smem_bytes<Key, Val>(cfg.class_cap[kNumClasses - 1])));
+      static int grid[kNumClasses] = {};
+      if (!grid[cls]) grid[cls] = grid_for(kern, ns, smem, di.sms);
+      const int g = grid[cls];
+      return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, ns, smem, s>>>(c, (uint32_t)cls); });
     }
-    if (phase == 0) return launch_small<CAP>(c, cfg, cls, di, s, prof, count, 0u);
-    return GSS_SUCCESS;
+    auto kern = k_small_block<Key, Val, IdT, Cmp>;
+    const size_t smem = block_sort_smem_bytes<Key, Val>(nt);
+    GSS_TRY(set_smem(kern, block_sort_smem_bytes<Key, Val>(kSmallMaxThreads)));
+    static int grid[kNumClasses + 1] = {};
+    if (!grid[cls]) grid[cls] = grid_for(kern, nt, smem, di.sms);
+    const int g = grid[cls];
+    return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, nt, smem, s>>>(c, (uint32_t)cls); });
   }
 
   // The whole launch sequence.  mode: sort / partition / partition_by.
@@ -360,23 +348,8 @@ struct Engine {
     }
     if (mode != MODE_SORT) return GSS_SUCCESS;
     // in-SM sorts, largest class first (buckets "ordered by size"; R8)
-    // phase 0: in-SM sample split + warp sorts; phase 1: block merge sort of the retries
-    for (int phase = 0; phase < 2; phase++) {
-      for (int cls = (int)cfg.nclass - 1; cls >= 0; cls--) {
-        switch (kClassCap[cls]) {
-          case 512: GSS_TRY(launch_class<512>(c, cfg, cls, di, s, prof, count, phase)); break;
-          case 1024: GSS_TRY(launch_class<1024>(c, cfg, cls, di, s, prof, count, phase)); break;
-          case 2048: GSS_TRY(launch_class<2048>(c, cfg, cls, di, s, prof, count, phase)); break;
-          case 4096: GSS_TRY(launch_class<4096>(c, cfg, cls, di, s, prof, count, phase)); break;
-          case 8192: GSS_TRY(launch_class<8192>(c, cfg, cls, di, s, prof, count, phase)); break;
-          case 16384:
-            if constexpr (max_small_capacity<Key, Val>() >= 16384) {
-              GSS_TRY(launch_class<16384>(c, cfg, cls, di, s, prof, count, phase));
-            }
-            break;
-        }
-      }
-    }
+    for (int cls = (int)cfg.nclass - 1; cls >= 0; cls--) GSS_TRY(launch_small(c, cfg, cls, di, s, prof, count));
+    if (cfg.flags & GSS_FLAG_SPLIT_SORT) GSS_TRY(launch_small(c, cfg, kNumClasses, di, s, prof, count));
     GSS_TRY(launch(prof, GSS_K_COPY, s, count, [&] { k_copy<Key, Val, IdT><<<di.sms * 4, 256, 0, s>>>(c); }));
     constexpr int NTO = 1024;
     auto ko = k_overflow<Key, Val, IdT, Cmp, NTO>;

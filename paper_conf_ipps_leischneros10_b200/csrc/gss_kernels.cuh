@@ -327,7 +327,10 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
 // so consecutive tiles mostly share a bucket and its tree stays in shared
 // memory.
 template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kClsThreads, 2) k_classify(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+#ifndef GSS_CLS_MINB
+#define GSS_CLS_MINB 2
+#endif
+__global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   constexpr uint32_t REP = rep_copies<Key>();
   Key* tree = reinterpret_cast<Key*>(smem_raw);
@@ -673,20 +676,19 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
   }
 }
 
-// Phase 4, default variant.  Every key takes its rank within (warp, chunk,
-// id) from one shared-memory atomic on its warp's counters (a warp whose 32
-// keys share an id -- sorted input -- takes one update for all of them), so
-// the result is deterministic though not stable (R7); a thread per id turns
-// the warp counts into warp starts, warp 0 scans the K chunk totals; the
-// chunk is reordered by id in shared memory and each bucket run is written
-// with coalesced stores.  CTA b handles the contiguous tile range [b*per,
-// (b+1)*per); the next chunk's keys, values and ids are loaded into registers
-// before the current chunk's runs are written out.
+// Phase 4, default variant (R7: a partition, not stable).  Every key takes
+// its rank within (chunk, id) from one shared-memory atomic on the CTA's
+// counter for its id; warp 0 scans the K chunk totals into staged run
+// offsets and staged -> global displacements; the chunk is reordered by id in
+// shared memory and each bucket run is written with coalesced stores.  One
+// counter set per CTA (not per warp) keeps the per-chunk bookkeeping at K
+// counters.  CTA b handles the contiguous tile range [b*per, (b+1)*per); the
+// next chunk's keys, values and ids are loaded into registers before the
+// current chunk's runs are written out.
 template <class Key, class Val, class IdT>
 struct ScatterFastSmem {
   static size_t bytes(uint32_t kmax) {
-    size_t b = (size_t)kmax * 4 * 4;                            // ctot, off, delta, gbase
-    b += (size_t)(kScatterThreads / 32) * kmax * 4;             // per-warp counters
+    size_t b = (size_t)kmax * 4 * 3;                            // cnt/off, delta, gbase
     b = (b + 15) & ~size_t(15);
     b += (size_t)kChunk * sizeof(Key);
     if (kHasVal<Val>) b += (size_t)kChunk * sizeof(Val);
@@ -699,13 +701,10 @@ template <class Key, class Val, class IdT, class Cmp>
 __global__ void __launch_bounds__(kScatterThreads, 2)
     k_scatter_fast(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  constexpr int NW = kScatterThreads / 32;
-  uint32_t* ctot = reinterpret_cast<uint32_t*>(smem_raw);
-  uint32_t* off = ctot + kmax;
-  uint32_t* delta = off + kmax;
+  uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw);          // chunk counts, then run offsets
+  uint32_t* delta = cnt + kmax;
   uint32_t* gbase = delta + kmax;
-  uint32_t* wcnt = gbase + kmax;                                   // NW x kmax
-  size_t o = ((size_t)kmax * 16 + (size_t)NW * kmax * 4 + 15) & ~size_t(15);
+  size_t o = ((size_t)kmax * 12 + 15) & ~size_t(15);
   Key* skeys = reinterpret_cast<Key*>(smem_raw + o);
   o += (size_t)kChunk * sizeof(Key);
   Val* svals = reinterpret_cast<Val*>(smem_raw + o);
@@ -722,8 +721,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
   if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
   const IdT* idsrc = c.ids;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  uint32_t* wc = wcnt + w * kmax;
-  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
+  const uint32_t cnt_s = (uint32_t)__cvta_generic_to_shared(cnt);
   const uint32_t q0 = w * (32 * kScatterIter) + lane;
   const uint32_t per = (nt + gridDim.x - 1) / gridDim.x;
   uint32_t t = blockIdx.x * per;
@@ -750,6 +748,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
   };
   tile_info(t);
   load_gbase();
+  for (uint32_t id = threadIdx.x; id < kmax; id += kScatterThreads) cnt[id] = 0;
   Key pk[kScatterIter];
   Val pv[kScatterIter];
   uint32_t pid[kScatterIter];
@@ -767,7 +766,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
   };
   uint32_t c0 = 0;
   load_chunk(beg, idb, min((uint32_t)kChunk, len));
-  __syncthreads();                                                 // gbase initialised
+  __syncthreads();                                                 // gbase and counters initialised
   for (;;) {
     const uint32_t clen = min((uint32_t)kChunk, len - c0);
     Key kk[kScatterIter];
@@ -779,38 +778,13 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
       iid[it] = pid[it];
       if constexpr (kHasVal<Val>) vv[it] = pv[it];
     }
-    // 1. ranks within (warp, id), from the warp's own counters: deterministic
-    //    (one warp's atomics are applied in a fixed order)
-    for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
-    __syncwarp();
+    // 1. rank within (chunk, id): one shared atomic per key on the CTA's counter
 #pragma unroll
-    for (int it = 0; it < kScatterIter; it++) {
-      const uint32_t id = iid[it];
-      const uint32_t first = __shfl_sync(kFull, id, 0);
-      if (__all_sync(kFull, id == first) && first != 0xffffffffu) {
-        uint32_t base = 0;
-        if (lane == 0) { base = wc[first]; wc[first] = base + 32u; }
-        __syncwarp();
-        rk[it] = __shfl_sync(kFull, base, 0) + (uint32_t)lane;
-      } else {
-        rk[it] = atom_add_shared_if(id != 0xffffffffu ? 1u : 0u, wc_s + 4 * (id & 0xffffu), 1u);
-      }
-    }
+    for (int it = 0; it < kScatterIter; it++)
+      rk[it] = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, cnt_s + 4 * (iid[it] & 0xffffu), 1u);
     __syncthreads();
-    // 2. per id: chunk total and every warp's start within the id's run
-    for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) {
-      uint32_t run = 0;
-#pragma unroll
-      for (int q = 0; q < NW; q++) {
-        const uint32_t x = wcnt[q * kmax + id];
-        wcnt[q * kmax + id] = run;
-        run += x;
-      }
-      ctot[id] = run;
-    }
-    __syncthreads();
-    // 3. warp 0: exclusive scan of the K chunk totals; staged position of id's
-    //    run (off) and staged -> global displacement (delta)
+    // 2. warp 0: exclusive scan of the K chunk totals -> staged run offsets
+    //    (cnt), staged -> global displacement (delta); gbase advances
     if (w == 0) {
       uint32_t run = 0;
       for (uint32_t id0 = 0; id0 < K; id0 += 32 * 8) {
@@ -818,7 +792,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
         uint32_t x[8], sum = 0;
 #pragma unroll
         for (int j = 0; j < 8; j++) {
-          x[j] = ib + j < K ? ctot[ib + j] : 0u;
+          x[j] = ib + j < K ? cnt[ib + j] : 0u;
           sum += x[j];
         }
         uint32_t inc = sum;
@@ -831,7 +805,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
 #pragma unroll
         for (int j = 0; j < 8; j++) {
           if (ib + j < K) {
-            off[ib + j] = ex;
+            cnt[ib + j] = ex;
             delta[ib + j] = gbase[ib + j] - ex;
             gbase[ib + j] += x[j];
           }
@@ -845,14 +819,14 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
       if (iid[it] != 0xffffffffu) {
-        const uint32_t pos = off[iid[it]] + wc[iid[it]] + rk[it];
+        const uint32_t pos = cnt[iid[it]] + rk[it];
         skeys[pos] = kk[it];
         if constexpr (kHasVal<Val>) svals[pos] = vv[it];
         sids[pos] = (IdT)iid[it];
       }
     }
     // advance and prefetch the next chunk (possibly of the next tile)
-    const uint32_t cur_clen = clen;
+    const uint32_t cur_clen = clen, cur_K = K;
     bool new_tile = false, done = false;
     c0 += kChunk;
     if (c0 >= len) {
@@ -863,20 +837,21 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
     }
     if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
     __syncthreads();
-    // 4. write this chunk's bucket runs
+    // 4. write this chunk's bucket runs; clear the counters for the next chunk
 #pragma unroll 4
     for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
       const uint32_t d = delta[sids[q]] + q;
       kdst[d] = skeys[q];
       if constexpr (kHasVal<Val>) vdst[d] = svals[q];
     }
+    for (uint32_t id = threadIdx.x; id < cur_K; id += kScatterThreads) cnt[id] = 0;
     if (done) break;
     if (new_tile) {
       // gbase is rewritten only after every thread has left step 4
       __syncthreads();
       load_gbase();
-      __syncthreads();
     }
+    __syncthreads();
   }
 }
 
@@ -1099,287 +1074,385 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
 // keys per thread of the bucket sorter (32 items per thread measured slower
 // on B200: register pressure outweighs the saved merge round), i.e. the
 // CtaSort default
-template <class Key, class Val, int CAP>
+template <class Key, class Val>
 constexpr int small_items() { return sort_items<Key, Val>(); }
-template <class Key, class Val, int CAP>
-constexpr int small_threads() { return CAP / small_items<Key, Val, CAP>(); }
+constexpr int kSmallMaxThreads = 1024;
 
-template <class Key, class Val, int CAP, int NT>
-constexpr int small_min_blocks() {
-  // 64 registers per thread (16 items), 128 with 32 items
-  return ((small_items<Key, Val, CAP>() >= 32 ? 512 : 1024) / NT) > 0 ? (small_items<Key, Val, CAP>() >= 32 ? 512 : 1024) / NT : 1;
+// ---------------------------------------------------------------------------
+// In-SM bucket sort, one CTA per bucket.  Both kernels below
+// serve every size class with one instantiation: the block has
+// class_warps(cls) warps (blockDim.x, chosen by the host).
+// ---------------------------------------------------------------------------
+
+// Block-wide merge sort: the bucket is loaded to shared memory, each thread
+// sorts ITEMS keys with the odd-even merge network, then merge-path rounds
+// across the whole CTA (CtaSort).  Used for the one-warp class (where it is
+// a warp sort), for the buckets the in-SM split hands back (cls ==
+// kNumClasses, 1024 threads), and for every class unless GSS_FLAG_SPLIT_SORT.
+template <class Key, class Val>
+__host__ __device__ constexpr size_t block_sort_smem_bytes(int nt) {
+  return (size_t)padded_len(nt * small_items<Key, Val>()) * (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0));
 }
 
-template <class Key, class Val, class IdT, class Cmp, int CAP, int NT = small_threads<Key, Val, CAP>()>
-__global__ void __launch_bounds__(NT, small_min_blocks<Key, Val, CAP, NT>())
-    k_small(Ctx<Key, Val, IdT> c, uint32_t cls, uint32_t retry) {
+template <class Key, class Val, class IdT, class Cmp>
+__global__ void __launch_bounds__(kSmallMaxThreads, 1)
+    k_small_block(Ctx<Key, Val, IdT> c, uint32_t cls) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  using Sorter = CtaSort<Key, Val, NT, Cmp, small_items<Key, Val, CAP>()>;
+  constexpr int ITEMS = small_items<Key, Val>();
+  using Sorter = CtaSort<Key, Val, kSmallMaxThreads, Cmp, ITEMS>;
+  const int nt = (int)blockDim.x;
   Key* sk = reinterpret_cast<Key*>(smem_raw);
-  Val* sv = reinterpret_cast<Val*>(smem_raw + (size_t)Sorter::PL * sizeof(Key));
+  Val* sv = reinterpret_cast<Val*>(smem_raw + (size_t)padded_len(nt * ITEMS) * sizeof(Key));
   const Cmp less;
-  const uint32_t ni = min(retry ? c.cnt->retry_count[cls] : c.cnt->small_count[cls], c.cap_small[cls]);
-  const Item* list = retry ? c.retry[cls] : c.small[cls];
+  const bool fb = cls == (uint32_t)kNumClasses;
+  const uint32_t ni = fb ? min(c.cnt->fb_count, c.cap_fb) : min(c.cnt->small_count[cls], c.cap_small[cls]);
+  const Item* list = fb ? c.fb : c.small[cls];
   for (uint32_t i = blockIdx.x; i < ni; i += gridDim.x) {
     const Item I = list[i];
-    // load the bucket with ITEMS independent loads in flight per thread
+    const uint32_t m = I.m;
     const Key* src = c.keys(I.buf) + I.lo;
     const Val* vs = nullptr;
     if constexpr (kHasVal<Val>) vs = c.vals(I.buf) + I.lo;
-    constexpr int LU = 4;                                  // loads in flight per thread
-    for (uint32_t q0 = threadIdx.x; q0 < I.m; q0 += LU * NT) {
+    // load the bucket with LU independent loads in flight per thread
+    constexpr int LU = 4;
+    for (uint32_t q0 = threadIdx.x; q0 < m; q0 += LU * nt) {
       Key tk[LU];
       Val tv[LU];
 #pragma unroll
       for (int u = 0; u < LU; u++) {
-        const uint32_t q = q0 + u * NT;
-        if (q < I.m) {
+        const uint32_t q = q0 + u * nt;
+        if (q < m) {
           tk[u] = src[q];
           if constexpr (kHasVal<Val>) tv[u] = vs[q];
         }
       }
 #pragma unroll
       for (int u = 0; u < LU; u++) {
-        const uint32_t q = q0 + u * NT;
-        if (q < I.m) {
+        const uint32_t q = q0 + u * nt;
+        if (q < m) {
           sk[phys(q)] = tk[u];
           if constexpr (kHasVal<Val>) sv[phys(q)] = tv[u];
         }
       }
     }
-    Sorter::sort(sk, sv, (int)I.m, less);
-    for (uint32_t q = threadIdx.x; q < I.m; q += NT) c.kout[I.lo + q] = sk[phys(q)];
+    Sorter::sort(sk, sv, (int)m, less, nt);
+    for (uint32_t q = threadIdx.x; q < m; q += nt) c.kout[I.lo + q] = sk[phys(q)];
     if constexpr (kHasVal<Val>)
-      for (uint32_t q = threadIdx.x; q < I.m; q += NT) c.vout[I.lo + q] = sv[phys(q)];
-    __syncthreads();
+      for (uint32_t q = threadIdx.x; q < m; q += nt) c.vout[I.lo + q] = sv[phys(q)];
+    if (nt == 32) __syncwarp(); else __syncthreads();
   }
 }
 
 // ---------------------------------------------------------------------------
-// In-SM bucket sort by one more sample-sort split inside shared memory
-// (the paper's "sample sort based" chunk sorter, re-derived for
-// B200): a warp sorts a sample of 4*k2 keys and takes k2-1 splitters; the
-// CTA classifies the bucket (Algorithm 2 descent in shared memory), counts,
-// and places every key into its sub-bucket's region of shared memory; then
-// each warp merge-sorts whole sub-buckets (odd-even merge network + merge
-// path) with warp barriers only and writes them to keys_out.
-// Equality sub-buckets (R4) need no sorting.  A sub-bucket larger than one
-// warp's capacity is written unsorted and retried by k_small.
+// GSS_FLAG_SPLIT_SORT (ablation) for classes of two or more warps: one more sample-sort split inside
+// the SM -- the paper's "sample sort based" chunk sorter,
+// re-derived for B200 -- so that no merge round ever spans more than one
+// warp (those rounds need a block barrier each and the longest merge-path
+// searches):
+//   B. warp 0 draws S = 128 (or 256) sample keys at hashed positions (R2,
+//      level tag 254), sorts them in registers (bitonic network, shuffles) and
+//      lays the k2 - 1 splitters out as the implicit tree
+//   C. every key (streamed from global memory) descends the tree
+//      (Algorithm 2; ties go left, R3); its sub-bucket id is kept
+//      in shared memory and the sub-bucket sizes are counted with shared atomics
+//   D. warp 0: sub-bucket offsets; consecutive sub-buckets are packed greedily
+//      into segments of at most WCAP keys (one warp's sort capacity), each
+//      starting at a 16-aligned shared slot
+//   E. every key (read again: L2 hits) takes the next slot of its sub-bucket
+//      (one shared atomic; the order inside a sub-bucket is irrelevant)
+//   F. each warp merge-sorts whole segments with warp barriers only and writes
+//      them out: sub-buckets are ordered ranges, so the concatenation of the
+//      sorted segments is the sorted bucket.
+// A sub-bucket larger than WCAP (heavy duplicates) or more than kMaxSegs
+// segments hands the bucket to k_small_block (the fb list).
 // ---------------------------------------------------------------------------
-constexpr int kSplitMaxK = 128;            // k2 <= 128 sub-buckets (K <= 255 ids)
-constexpr int kSplitPad = 256;             // per-region padding slack (one per id)
+constexpr int kSubMaxK = 256;            // sub-buckets per bucket (power of two; ids are u8)
+constexpr int kMaxSegs = 128;            // warp segments per bucket
+constexpr int kSegSlack = 16 * kMaxSegs; // alignment slack (slots)
 
-template <class Key, class Val, int CAP, int NT>
-struct SplitSortSmem {
-  static constexpr int NW = NT / 32;
-  static constexpr int PL = padded_len(CAP) + kSplitPad + 16;
-  __host__ __device__ static constexpr size_t off_vals() { return (size_t)PL * sizeof(Key); }
-  __host__ __device__ static constexpr size_t off_ids() { return off_vals() + (kHasVal<Val> ? (size_t)PL * sizeof(Val) : 0); }
-  __host__ __device__ static constexpr size_t off_tree() { return (off_ids() + CAP + 15) & ~size_t(15); }
-  __host__ __device__ static constexpr size_t off_spl() { return off_tree() + kSplitMaxK * sizeof(Key); }
-  __host__ __device__ static constexpr size_t off_wcnt() { return off_spl() + kSplitMaxK * sizeof(Key); }
-  __host__ __device__ static constexpr size_t off_tot() { return off_wcnt() + (size_t)NW * 256 * 4; }
-  __host__ __device__ static constexpr size_t off_cst() { return off_tot() + 256 * 4; }
-  __host__ __device__ static constexpr size_t off_rst() { return off_cst() + 256 * 4; }
-  __host__ __device__ static constexpr size_t off_misc() { return off_rst() + 256 * 4; }
-  __host__ __device__ static constexpr size_t bytes() { return off_misc() + 16 * 4; }
-};
+// keys per lane of the segment sorter: 16 for 4-byte keys, else 8 (64 registers)
+#ifndef GSS_SEG_ITEMS_WIDE
+#define GSS_SEG_ITEMS_WIDE 16
+#endif
+template <class Key, class Val>
+constexpr int seg_items() { return (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0)) > 8 ? 8 : GSS_SEG_ITEMS_WIDE; }
 
-template <class Key, class Val, int CAP>
-constexpr int split_threads() { return 256; }
-
-// Warp-level sorts called out of line (keeps the split kernel's registers low).
-template <class Key, class Val, class Cmp, int ITEMS>
-__device__ __forceinline__ void warp_sort(Key* rk, Val* rv, int t) {
-  CtaSort<Key, Val, 32, Cmp, ITEMS>::sort(rk, rv, t, Cmp());
+// Dynamic shared memory of the split sorter for a class of capacity cap:
+// key (+ value) slots plus alignment slack, and one u8 sub-bucket id per key.
+template <class Key, class Val>
+__host__ __device__ constexpr size_t small_smem_bytes(uint32_t cap) {
+  return (size_t)padded_len((int)cap + kSegSlack) * (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0)) + cap;
 }
 
-template <class Key, class Val, class IdT, class Cmp, int CAP, int NT = split_threads<Key, Val, CAP>()>
-__global__ void __launch_bounds__(NT, 2) k_split_sort(Ctx<Key, Val, IdT> c, uint32_t cls) {
+// Bitonic sort of 32 * P keys held P per lane in registers (lane l holds
+// sorted positions l*P .. l*P + P - 1 afterwards): in-lane compare-exchanges
+// for strides < P, shuffles across lanes for the others.  Used for the
+// split's sample (the sample sort "fits in shared memory", P:347-349 --
+// here it fits in one warp's registers).
+template <int P, class Key, class Cmp>
+__device__ __forceinline__ void warp_bitonic_sort(Key (&x)[P], Cmp less) {
+  const int lane = threadIdx.x & 31;
+#pragma unroll
+  for (int k = 2; k <= 32 * P; k <<= 1) {
+#pragma unroll
+    for (int j = k >> 1; j > 0; j >>= 1) {
+      if (j >= P) {
+        const int lj = j / P;
+        const bool lower = (lane & lj) == 0;
+#pragma unroll
+        for (int i = 0; i < P; i++) {
+          const bool up = ((lane * P + i) & k) == 0;
+          const Key y = __shfl_xor_sync(kFull, x[i], lj);
+          const bool take = (lower == up) ? less(y, x[i]) : less(x[i], y);
+          x[i] = take ? y : x[i];
+        }
+      } else {
+#pragma unroll
+        for (int i = 0; i < P; i++) {
+          if ((i & j) == 0) {
+            const bool up = ((lane * P + i) & k) == 0;
+            const bool sw = up ? less(x[i + j], x[i]) : less(x[i], x[i + j]);
+            const Key a = sw ? x[i + j] : x[i], b = sw ? x[i] : x[i + j];
+            x[i] = a;
+            x[i + j] = b;
+          }
+        }
+      }
+    }
+  }
+}
+
+// Warp 0 of the split: S = 32 * P sample keys at hashed positions (R2, level
+// tag 254), sorted in registers; splitter i = S[(i + 1) * S / k2] goes to
+// node j of the implicit tree (D1) via a shared staging array.
+template <int P, class Key, class Cmp>
+__device__ __forceinline__ void split_splitters(const Key* src, uint64_t seed, uint64_t lo, uint32_t m, uint32_t k2,
+                                                Key* stage, Key* tree) {
+  const int lane = threadIdx.x & 31;
+  Key x[P];
+#pragma unroll
+  for (int i = 0; i < P; i++) x[i] = src[sample_pos(seed, 254, lo, (uint64_t)(lane * P + i), m)];
+  warp_bitonic_sort<P>(x, Cmp());
+#pragma unroll
+  for (int i = 0; i < P; i++) stage[lane * P + i] = x[i];
+  __syncwarp();
+  const uint32_t r = (32u * P) / k2;                      // oversampling
+  for (uint32_t j = lane + 1; j < k2; j += 32) {
+    const uint32_t d = ilog2(j), q = j - (1u << d);
+    const uint32_t si = ((2 * q + 1) * k2) >> (d + 1);    // splitter index + 1
+    tree[j] = stage[si * r];
+  }
+}
+
+template <class Key>
+struct SmallSplitShared {
+  Key tree[kSubMaxK];                    // tree[1 .. k2-1]
+  uint32_t cnt[kSubMaxK];                // sub-bucket sizes, then slot cursors
+  uint32_t pre[kSubMaxK + 1];            // exclusive prefix of the sizes
+  uint32_t nxt[kSubMaxK];                // greedy packing: first sub-bucket after a segment started here
+  int32_t mark[kSubMaxK];                // segment index at a segment's first sub-bucket, else -1
+  uint32_t seg_smem[kMaxSegs], seg_out[kMaxSegs], seg_len[kMaxSegs];
+  uint32_t nseg, fallback;
+};
+
+// At most kSplitMaxThreads threads: the 16-key-per-lane segment sort of
+// 8-byte keys needs about 72 registers; larger classes get more segments
+// per warp (the keys are streamed, so the block size is free).
+constexpr int kSplitMaxThreads = 448;
+
+template <class Key, class Val, class IdT, class Cmp>
+__global__ void __launch_bounds__(kSplitMaxThreads, 2)
+    k_small(Ctx<Key, Val, IdT> c, uint32_t cls) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  using L = SplitSortSmem<Key, Val, CAP, NT>;
-  using WSort = CtaSort<Key, Val, 32, Cmp>;                 // one warp: 32*ITEMS keys
-  using WSort4 = CtaSort<Key, Val, 32, Cmp, 4>;             // smaller sub-buckets: all lanes busy
-  using WSort8 = CtaSort<Key, Val, 32, Cmp, 8>;
-  constexpr int NW = NT / 32;
-  constexpr int WCAP = WSort::C;
+  __shared__ SmallSplitShared<Key> sh;
+  constexpr int ITEMS = small_items<Key, Val>();
+  constexpr int WITEMS = seg_items<Key, Val>();
+  constexpr uint32_t WCAP = 32 * WITEMS;                   // one warp's sort capacity
+  constexpr uint32_t kSubMean = WCAP / 4;                  // target keys per sub-bucket
+  using WSort = CtaSort<Key, Val, 32, Cmp, WITEMS>;
+  const int nt = (int)blockDim.x;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, nw = nt >> 5;
+  const uint32_t cap = c.class_cap[cls];
+  const size_t slots = (size_t)padded_len((int)cap + kSegSlack);
   Key* sk = reinterpret_cast<Key*>(smem_raw);
-  Val* sv = reinterpret_cast<Val*>(smem_raw + L::off_vals());
-  uint8_t* sid = smem_raw + L::off_ids();
-  Key* tree = reinterpret_cast<Key*>(smem_raw + L::off_tree());
-  Key* spl = reinterpret_cast<Key*>(smem_raw + L::off_spl());
-  uint32_t* wcnt = reinterpret_cast<uint32_t*>(smem_raw + L::off_wcnt());
-  uint32_t* tot = reinterpret_cast<uint32_t*>(smem_raw + L::off_tot());
-  uint32_t* cst = reinterpret_cast<uint32_t*>(smem_raw + L::off_cst());
-  uint32_t* rst = reinterpret_cast<uint32_t*>(smem_raw + L::off_rst());
-  uint32_t* misc = reinterpret_cast<uint32_t*>(smem_raw + L::off_misc());
+  Val* sv = reinterpret_cast<Val*>(smem_raw + slots * sizeof(Key));
+  uint8_t* sid = smem_raw + slots * (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0));
   const Cmp less;
-  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
-  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + w * 256);
   const uint32_t ni = min(c.cnt->small_count[cls], c.cap_small[cls]);
-  for (uint32_t it = blockIdx.x; it < ni; it += gridDim.x) {
-    const Item I = c.small[cls][it];
+  const Item* list = c.small[cls];
+  for (uint32_t i = blockIdx.x; i < ni; i += gridDim.x) {
+    const Item I = list[i];
     const uint32_t m = I.m;
     const Key* src = c.keys(I.buf) + I.lo;
-    const Val* vsrc = nullptr;
-    if constexpr (kHasVal<Val>) vsrc = c.vals(I.buf) + I.lo;
-    Key* kout = c.kout + I.lo;
-    Val* vout = nullptr;
-    if constexpr (kHasVal<Val>) vout = c.vout + I.lo;
-    // ---- 1. sample and splitters (warp 0); the other warps clear counters
-    uint32_t k2 = 2;                                   // sub-buckets of about WCAP/4 keys
-    while (k2 < kSplitMaxK && k2 * (WCAP / 4) < m) k2 <<= 1;
-    const uint32_t s = 4 * k2;
-    for (uint32_t j = threadIdx.x; j < (uint32_t)NW * 256; j += NT) wcnt[j] = 0;
-    if (w == 0) {
-      for (uint32_t j = lane; j < s; j += 32) sk[phys(j)] = src[sample_pos(c.seed, 254, I.lo, j, m)];
-      if (s <= 128) warp_sort<Key, NoVal, Cmp, 4>(sk, nullptr, (int)s);
-      else if (s <= 256) warp_sort<Key, NoVal, Cmp, 8>(sk, nullptr, (int)s);
-      else warp_sort<Key, NoVal, Cmp, 16>(sk, nullptr, (int)s);
-      bool dup = false;
-      for (uint32_t i = lane; i + 2 < k2; i += 32) dup |= !less(sk[phys(4 * (i + 1) - 1)], sk[phys(4 * (i + 2) - 1)]);
-      const bool eq = __any_sync(kFull, dup) || k2 == 2;
-      const uint32_t ks = eq ? max(2u, k2 / 2) : k2;
-      const uint32_t stride = s / ks;
-      for (uint32_t i = lane; i + 1 < ks; i += 32) spl[i] = sk[phys(stride * (i + 1) - 1)];
-      for (uint32_t j = lane + 1; j < ks; j += 32) {
-        const uint32_t d = ilog2(j), q = j - (1u << d);
-        tree[j] = sk[phys(stride * (((2 * q + 1) * ks) >> (d + 1)) - 1)];
-      }
-      if (lane == 0) { misc[0] = ks; misc[1] = eq ? 1u : 0u; misc[2] = eq ? 2 * ks - 1 : ks; misc[3] = 0; }
+    const Val* vs = nullptr;
+    if constexpr (kHasVal<Val>) vs = c.vals(I.buf) + I.lo;
+    // ---- A. clear the sub-bucket tables
+    uint32_t k2 = 2;
+    while (k2 < (uint32_t)kSubMaxK && k2 * kSubMean < m) k2 <<= 1;
+    for (uint32_t j = threadIdx.x; j < k2; j += nt) {
+      sh.cnt[j] = 0;
+      sh.mark[j] = -1;
+    }
+    // ---- B. warp 0: sample, sort it in registers, splitter tree
+    if (warp == 0) {
+      if (k2 <= 128) split_splitters<4, Key, Cmp>(src, c.seed, I.lo, m, k2, sk, sh.tree);
+      else split_splitters<8, Key, Cmp>(src, c.seed, I.lo, m, k2, sk, sh.tree);
     }
     __syncthreads();
-    const uint32_t ks = misc[0], K = misc[2];
-    const bool eq = misc[1] != 0;
-    const uint32_t logk = ilog2(ks);
-    // ---- 2. classify every key, count per warp (striped: q = r*NT + tid)
+    // ---- C. descend (Algorithm 2), count, keep the id (keys streamed from
+    // global memory, GR per thread in flight; no keys held across barriers)
     {
-      constexpr uint32_t W = sizeof(Key);
-      constexpr int U = 8;
-      const uint32_t step0 = 0u - tree_s, step1 = W - tree_s;
-      for (uint32_t q0 = threadIdx.x; q0 < m; q0 += U * NT) {
-        Key e[U];
-        uint32_t a[U];
+      const uint32_t logk = ilog2(k2);
+      constexpr int GR = 4;
+      for (uint32_t q0 = threadIdx.x; q0 < m; q0 += GR * nt) {
+        Key e[GR];
+        uint32_t jj[GR];
 #pragma unroll
-        for (int u = 0; u < U; u++) {
-          a[u] = tree_s + W;
-          if (q0 + u * NT < m) e[u] = src[q0 + u * NT];
+        for (int u = 0; u < GR; u++) {
+          const uint32_t q = q0 + u * nt;
+          if (q < m) e[u] = src[q];
+          jj[u] = 1;
         }
         for (uint32_t d = 0; d < logk; d++) {
 #pragma unroll
-          for (int u = 0; u < U; u++) a[u] = a[u] + a[u] + (less(ld_shared<Key>(a[u]), e[u]) ? step1 : step0);
+          for (int u = 0; u < GR; u++) jj[u] = 2 * jj[u] + (less(sh.tree[jj[u]], e[u]) ? 1u : 0u);
         }
 #pragma unroll
-        for (int u = 0; u < U; u++) {
-          const uint32_t q = q0 + u * NT;
+        for (int u = 0; u < GR; u++) {
+          const uint32_t q = q0 + u * nt;
           if (q < m) {
-            uint32_t id = (a[u] - tree_s) / W - ks;
-            if (eq) id = 2 * id + ((id + 1 < ks && !less(e[u], spl[id])) ? 1u : 0u);
+            const uint32_t id = jj[u] - k2;
             sid[q] = (uint8_t)id;
-            red_shared_add(wc_s + 4 * id, 1u);
+            red_shared_add((uint32_t)__cvta_generic_to_shared(&sh.cnt[id]), 1u);
           }
         }
       }
     }
     __syncthreads();
-    // ---- 3. sub-bucket sizes, output offsets, padded shared regions, warp cursors
-    if (threadIdx.x < K) {
-      uint32_t t = 0;
-#pragma unroll 4
-      for (int q = 0; q < NW; q++) t += wcnt[q * 256 + threadIdx.x];
-      tot[threadIdx.x] = t;
-    }
-    __syncthreads();
-    if (w == 0) {
-      // K <= 255: one warp scans sizes and padded region sizes
-      uint32_t run_c = 0, run_r = 0;
-      for (uint32_t j0 = 0; j0 < K; j0 += 32) {
-        const uint32_t j = j0 + lane;
-        const uint32_t t = j < K ? tot[j] : 0u;
-        const uint32_t pr = t ? (uint32_t)padded_len((int)t) : 0u;
-        uint32_t ic = t, ir = pr;
+    // ---- D. offsets, greedy segments, slot cursors (warp 0; lane l owns
+    // sub-buckets [l*PER, l*PER + PER))
+    if (warp == 0) {
+      constexpr int PER = kSubMaxK / 32;
+      const uint32_t j0 = lane * PER, j1 = min(j0 + PER, k2);
+      uint32_t sum = 0, mx = 0;
+#pragma unroll 1
+      for (uint32_t j = j0; j < j1; j++) { const uint32_t x = sh.cnt[j]; sum += x; mx = max(mx, x); }
+      uint32_t incl = sum;
 #pragma unroll
-        for (int o = 1; o < 32; o <<= 1) {
-          const uint32_t yc = __shfl_up_sync(kFull, ic, o), yr = __shfl_up_sync(kFull, ir, o);
-          if (lane >= o) { ic += yc; ir += yr; }
-        }
-        if (j < K) { cst[j] = run_c + ic - t; rst[j] = run_r + ir - pr; }
-        run_c += __shfl_sync(kFull, ic, 31);
-        run_r += __shfl_sync(kFull, ir, 31);
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(kFull, incl, o);
+        if (lane >= o) incl += y;
       }
-    }
-    __syncthreads();
-    if (threadIdx.x < K) {
-      const uint32_t j = threadIdx.x;
-      uint32_t run = 0;
-      for (int q = 0; q < NW; q++) {
-        const uint32_t x = wcnt[q * 256 + j];
-        wcnt[q * 256 + j] = run;
-        run += x;
-      }
-    }
-    __syncthreads();
-    // ---- 4. place every key in its sub-bucket region (same striping as step 2)
-    {
-      constexpr int U = 8;
-      for (uint32_t q0 = threadIdx.x; q0 < m; q0 += U * NT) {
-        Key e[U];
-        Val v[U];
-#pragma unroll
-        for (int u = 0; u < U; u++) {
-          const uint32_t q = q0 + u * NT;
-          if (q < m) {
-            e[u] = src[q];
-            if constexpr (kHasVal<Val>) v[u] = vsrc[q];
+      uint32_t run = incl - sum;
+#pragma unroll 1
+      for (uint32_t j = j0; j < j1; j++) { sh.pre[j] = run; run += sh.cnt[j]; }
+      if (lane == 0) sh.pre[k2] = m;
+      mx = warp_max32(mx);
+      __syncwarp();
+      bool fb = mx > WCAP;
+      if (!fb) {
+#pragma unroll 1
+        for (uint32_t j = j0; j < j1; j++) {
+          const uint32_t target = sh.pre[j] + WCAP;
+          uint32_t lo = j + 1, hi = k2;                    // largest e with pre[e] <= target
+          while (lo < hi) {
+            const uint32_t mid = (lo + hi + 1) >> 1;
+            if (sh.pre[mid] <= target) lo = mid; else hi = mid - 1;
           }
+          sh.nxt[j] = lo;
         }
-#pragma unroll
-        for (int u = 0; u < U; u++) {
-          const uint32_t q = q0 + u * NT;
-          if (q < m) {
-            const uint32_t id = sid[q];
-            uint32_t r;
-            asm volatile("atom.shared.add.u32 %0, [%1], 1;" : "=r"(r) : "r"(wc_s + 4 * id));
-            const uint32_t pos = rst[id] + (uint32_t)phys((int)r);
-            sk[pos] = e[u];
-            if constexpr (kHasVal<Val>) sv[pos] = v[u];
-          }
-        }
-      }
-    }
-    __syncthreads();
-    // ---- 5. warps take whole sub-buckets: sort and write out
-    for (;;) {
-      uint32_t j = 0;
-      if (lane == 0) j = atomicAdd(&misc[3], 1u);
-      j = __shfl_sync(kFull, j, 0);
-      if (j >= K) break;
-      const uint32_t t = tot[j];
-      if (t == 0) continue;
-      Key* rk = sk + rst[j];
-      Val* rv = nullptr;
-      if constexpr (kHasVal<Val>) rv = sv + rst[j];
-      const bool needs_sort = t > 1 && !(eq && (j & 1));
-      if (needs_sort && t > (uint32_t)WCAP) {
-        // too large for one warp: write unsorted, retry with the block merge sort
+        __syncwarp();
         if (lane == 0) {
-          uint32_t rc = 0;
-          while (rc + 1 < kNumClasses && t > c.class_cap[rc]) rc++;
-          const uint32_t slot = atomicAdd(&c.cnt->retry_count[rc], 1u);
-          if (slot < c.cap_small[rc]) c.retry[rc][slot] = Item{I.lo + cst[j], t, BUF_OUT, 0};
+          uint32_t sb = 0, n = 0, slot = 0;
+          while (sb < k2 && n < (uint32_t)kMaxSegs) {
+            const uint32_t e = sh.nxt[sb];
+            const uint32_t len = sh.pre[e] - sh.pre[sb];
+            sh.seg_smem[n] = slot; sh.seg_out[n] = sh.pre[sb]; sh.seg_len[n] = len;
+            sh.mark[sb] = (int32_t)n;
+            slot += (len + 15u) & ~15u;
+            n++;
+            sb = e;
+          }
+          sh.nseg = n;
+          sh.fallback = sb < k2 ? 1u : 0u;
+        }
+        __syncwarp();
+        fb = sh.fallback != 0;
+      }
+      if (fb) {
+        if (lane == 0) {
+          sh.fallback = 1;
+          const uint32_t slot = atomicAdd(&c.cnt->fb_count, 1u);
+          if (slot < c.cap_fb) c.fb[slot] = I;
           else atomicOr(&c.cnt->err, 16u);
         }
-      } else if (needs_sort) {
-        if (t <= (uint32_t)WSort4::C && WSort4::C < WCAP) warp_sort<Key, Val, Cmp, 4>(rk, rv, (int)t);
-        else if (t <= (uint32_t)WSort8::C && WSort8::C < WCAP) warp_sort<Key, Val, Cmp, 8>(rk, rv, (int)t);
-        else warp_sort<Key, Val, Cmp, WSort::ITEMS>(rk, rv, (int)t);
+      } else {
+        // segment of sub-bucket j = the last mark at or before j (prefix max)
+        int32_t gm = -1;
+#pragma unroll 1
+        for (uint32_t j = j0; j < j1; j++) gm = max(gm, sh.mark[j]);
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+          const int32_t y = __shfl_up_sync(kFull, gm, o);
+          if (lane >= o) gm = max(gm, y);
+        }
+        int32_t g = __shfl_up_sync(kFull, gm, 1);
+        if (lane == 0) g = -1;
+#pragma unroll 1
+        for (uint32_t j = j0; j < j1; j++) {
+          g = max(g, sh.mark[j]);
+          sh.cnt[j] = sh.seg_smem[g] + sh.pre[j] - sh.seg_out[g];
+        }
       }
-      for (uint32_t r = lane; r < t; r += 32) {
-        kout[cst[j] + r] = rk[phys((int)r)];
-        if constexpr (kHasVal<Val>) vout[cst[j] + r] = rv[phys((int)r)];
+    }
+    __syncthreads();
+    if (sh.fallback) {                                     // k_small_block sorts it later
+      __syncthreads();
+      continue;
+    }
+    // ---- E. every key (and value) takes the next slot of its sub-bucket
+    {
+      constexpr int GR = 4;
+      for (uint32_t q0 = threadIdx.x; q0 < m; q0 += GR * nt) {
+        Key e[GR];
+        Val v[GR];
+#pragma unroll
+        for (int u = 0; u < GR; u++) {
+          const uint32_t q = q0 + u * nt;
+          if (q < m) {
+            e[u] = src[q];
+            if constexpr (kHasVal<Val>) v[u] = vs[q];
+          }
+        }
+#pragma unroll
+        for (int u = 0; u < GR; u++) {
+          const uint32_t q = q0 + u * nt;
+          if (q < m) {
+            const uint32_t pos = atomicAdd(&sh.cnt[sid[q]], 1u);
+            sk[phys(pos)] = e[u];
+            if constexpr (kHasVal<Val>) sv[phys(pos)] = v[u];
+          }
+        }
       }
-      __syncwarp();
+    }
+    __syncthreads();
+    // ---- F. warps sort whole segments and write them out
+    {
+      Key* kout = c.kout + I.lo;
+      Val* vout = nullptr;
+      if constexpr (kHasVal<Val>) vout = c.vout + I.lo;
+      const uint32_t nseg = sh.nseg;
+      for (uint32_t g = warp; g < nseg; g += nw) {
+        const uint32_t base = sh.seg_smem[g], len = sh.seg_len[g], out = sh.seg_out[g];
+        Key* gk = sk + phys(base);                         // base is 16-aligned: phys(base + r) = phys(base) + phys(r)
+        Val* gv = nullptr;
+        if constexpr (kHasVal<Val>) gv = sv + phys(base);
+        if (len > 1) WSort::sort(gk, gv, (int)len, less);
+        for (uint32_t r = lane; r < len; r += 32) {
+          kout[out + r] = gk[phys(r)];
+          if constexpr (kHasVal<Val>) vout[out + r] = gv[phys(r)];
+        }
+      }
     }
     __syncthreads();
   }

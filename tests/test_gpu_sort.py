@@ -36,6 +36,12 @@ def oracle_params(oracle_mod, k=256, M=16384, a=30, seed=5489, k_policy="adaptiv
                              sample_cap=16384, seed=seed)
 
 
+def _few(n, width):
+    """3 distinct keys (test-side input shape, no method arithmetic)."""
+    x = inputs.keys("uniform", n, width, seed=4)
+    return (x % x.dtype.type(3)) * x.dtype.type(1000003)
+
+
 def check_pairs(x, v_out, k_out):
     n = x.size
     vo = v_out.astype(np.int64)
@@ -215,17 +221,41 @@ def test_full_size(gss, oracle_mod, width, n, dist):
 
 
 @pytest.mark.parametrize("width,pairs", KINDS)
-@pytest.mark.parametrize("dist", ["uniform", "dd", "and3", "equal"])
-def test_split_sort_variant(gss, width, pairs, dist):
-    """The in-SM sample-split bucket sorter (GSS_FLAG_SPLIT_SORT) gives the same keys."""
+@pytest.mark.parametrize("dist", ["uniform", "dd", "and3", "equal", "few"])
+@pytest.mark.parametrize("flags", [0, 2])
+def test_bucket_sorter_variants(gss, oracle_mod, width, pairs, dist, flags):
+    """Both bucket sorters give the oracle's keys: the CTA-wide merge sort
+    (default) and the in-SM sample split + warp segment sorts
+    (GSS_FLAG_SPLIT_SORT = 2).  'few' (3 distinct keys) drives every bucket of
+    the split into its hand-back path (a sub-bucket larger than a warp)."""
     n = (1 << 19) + 77
-    x = inputs.keys(dist, n, width, seed=2)
+    x = _few(n, width) if dist == "few" else inputs.keys(dist, n, width, seed=2)
     v = inputs.values(n, width) if pairs else None
-    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=2, stats=True)
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=flags, stats=True)
     assert st.error_flags == 0
-    np.testing.assert_array_equal(to_host(ko), np.sort(x))
+    want = oracle_mod.sort(x, None, oracle_params(oracle_mod))[0]
+    np.testing.assert_array_equal(to_host(ko), want)
     if pairs:
-        check_pairs(x, to_host(vo), np.sort(x))
+        check_pairs(x, to_host(vo), want)
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("m", [513, 4097, 9000, 16384])
+@pytest.mark.parametrize("flags", [0, 2])
+def test_single_bucket(gss, oracle_mod, width, pairs, m, flags):
+    """n <= M: the whole input is one in-SM bucket (no distribution level), sorted
+    by the bucket sorter of its size class; sizes straddle class boundaries."""
+    cap = 8192 if (pairs and width == 64) else 16384
+    m = min(m, cap)
+    for dist in ("uniform", "few"):
+        x = _few(m, width) if dist == "few" else inputs.keys(dist, m, width, seed=3)
+        v = inputs.values(m, width) if pairs else None
+        ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=flags, stats=True)
+        assert st.error_flags == 0 and st.levels == 0
+        want = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=cap))[0]
+        np.testing.assert_array_equal(to_host(ko), want)
+        if pairs:
+            check_pairs(x, to_host(vo), want)
 
 
 def test_distributed_sorter_single_rank_nccl(gss):
