@@ -221,6 +221,22 @@ __device__ __forceinline__ uint64_t block_sum_u64(uint64_t x, unsigned long long
 __host__ __device__ constexpr int padded_len(int c) { return c + c / 16 + 1; }
 __device__ __forceinline__ int phys(int i) { return i + (i >> 4); }
 
+// sk[phys(i)] as a volatile shared load: issued unconditionally (the
+// compiler may not turn a select on its result into a branch around it)
+template <class T>
+__device__ __forceinline__ T lds_key(const T* sk, int i) {
+  const uint32_t s = (uint32_t)__cvta_generic_to_shared(sk + phys(i));
+  if constexpr (sizeof(T) == 8) {
+    unsigned long long x;
+    asm volatile("ld.volatile.shared.u64 %0, [%1];" : "=l"(x) : "r"(s));
+    return bit_cast_dev<T>(x);
+  } else {
+    uint32_t x;
+    asm volatile("ld.volatile.shared.u32 %0, [%1];" : "=r"(x) : "r"(s));
+    return bit_cast_dev<T>(x);
+  }
+}
+
 // a = *p if pred, else b = *p: one predicated shared-memory load per target
 template <class T>
 __device__ __forceinline__ void load_pred(T& a, T& b, const T* p, bool pred) {
@@ -368,22 +384,34 @@ struct CtaSort {
                                                      int diag, Key* k, Val* v, Cmp less) {
     const int bEnd = ps + aLen + bLen - 1;                   // B's smallest key
     int ia;
+    // Merge-path search as binary lifting with a fixed number of steps (the
+    // pair width w = max(aLen, ...) is a power of two, the same for every lane
+    // of the round): no data-dependent trip count, no divergence.
+    const int w = aLen;                                       // aLen == w for every pair with a B run
     if constexpr (KV) {
-      // number of A keys among the first diag outputs, A first on ties
-      int lo = max(0, diag - bLen), hi = min(diag, aLen);
-      while (lo < hi) {
-        const int mid = (lo + hi) >> 1;
-        if (less(sk[phys(bEnd - (diag - 1 - mid))], sk[phys(ps + mid)])) hi = mid; else lo = mid + 1;
+      // number of A keys among the first diag outputs, A first on ties:
+      // smallest j in [lo, hi) with B[diag-1-j] < A[j], else hi
+      const int lo = max(0, diag - bLen), hi = min(diag, aLen);
+      int j = lo;
+      for (int st = w; st > 0; st >>= 1) {
+        const int pr = j + st - 1;
+        const int pc = min(pr, hi - 1);                     // clamped probe: the loads stay inside the pair
+        const Key b = lds_key(sk, bEnd - (diag - 1 - pc)), a = lds_key(sk, ps + pc);
+        j = (pr < hi) & !less(b, a) ? pr + 1 : j;
       }
-      ia = lo;
+      ia = j;
     } else {
-      // number of B keys among the first diag outputs, B first on ties
-      int lo = max(0, diag - aLen), hi = min(diag, bLen);
-      while (lo < hi) {
-        const int mid = (lo + hi) >> 1;
-        if (less(sk[phys(ps + diag - 1 - mid)], sk[phys(bEnd - mid)])) hi = mid; else lo = mid + 1;
+      // number of B keys among the first diag outputs, B first on ties:
+      // smallest j in [lo, hi) with A[diag-1-j] < B[j], else hi
+      const int lo = max(0, diag - aLen), hi = min(diag, bLen);
+      int j = lo;
+      for (int st = w; st > 0; st >>= 1) {
+        const int pr = j + st - 1;
+        const int pc = min(pr, hi - 1);                     // clamped probe (at most one slot past the pair)
+        const Key a = lds_key(sk, ps + diag - 1 - pc), b = lds_key(sk, bEnd - pc);
+        j = (pr < hi) & !less(a, b) ? pr + 1 : j;
       }
-      ia = diag - lo;
+      ia = diag - j;
     }
     int xa = ps + ia, xb = bEnd - (diag - ia);
     const int ae = ps + aLen;
