@@ -34,7 +34,7 @@ struct gss_profiler {
 namespace gssh {
 
 inline constexpr uint32_t kVersion = 1;
-inline constexpr uint32_t kFlagScatterFast = 1u << 30;   // experimental scatter variant (k_scatter_fast)
+inline constexpr uint32_t kFlagScatterWarpCounters = 1u << 30;   // ablation: unstable ranks from per-warp counters (k_scatter)
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -335,9 +335,11 @@ struct Engine {
                      [&] { k_scan_reduce<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
       GSS_TRY(launch(prof, GSS_K_SCAN, s, count,
                      [&] { k_scan_final<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
-      if (c.stable || !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterFast))) {
+      // stable ranks (R7 probe, GSS_FLAG_STABLE) and the per-warp-counter ablation: k_scatter;
+      // default: k_scatter_fast (one counter set per CTA); the paper's direct scatter: k_scatter_direct
+      if (c.stable || (cfg.flags & kFlagScatterWarpCounters)) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));
-      } else if (cfg.flags & kFlagScatterFast) {
+      } else if (!(cfg.flags & GSS_FLAG_DIRECT_SCATTER)) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksf<<<g_sf, kScatterThreads, sm_sf, s>>>(c, l, kmax); }));
       } else {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count,

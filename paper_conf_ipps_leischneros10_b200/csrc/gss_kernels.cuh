@@ -15,7 +15,13 @@
 namespace gss {
 
 constexpr int kClsThreads = 256;
-constexpr int kScatterThreads = 512;
+#ifndef GSS_SCATTER_THREADS
+#define GSS_SCATTER_THREADS 512
+#endif
+#ifndef GSS_SCATTER_MINB
+#define GSS_SCATTER_MINB 2
+#endif
+constexpr int kScatterThreads = GSS_SCATTER_THREADS;
 constexpr int kScatterIter = 8;                                   // keys per thread per chunk
 constexpr int kChunk = kScatterThreads * kScatterIter;            // 4096 keys staged per chunk
 constexpr int kScanCtas = 256;
@@ -478,7 +484,7 @@ __device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t s
 // into registers before the current chunk's runs are written out, so the
 // global-load latency overlaps the write phase and the barriers.
 template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+__global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   constexpr int NW = kScatterThreads / 32;
   uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);
@@ -687,20 +693,27 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter(Ctx<Key, Val, Id
 // current chunk's runs are written out.
 template <class Key, class Val, class IdT>
 struct ScatterFastSmem {
+  // staging of the current chunk's keys in natural order frees their
+  // registers for the next chunk's loads (not for 16-byte pairs: smem)
+#ifndef GSS_SCATTER_STAGE
+#define GSS_SCATTER_STAGE 0      // staging measured slower on B200 (3.40 vs 3.13 ms per 2^28 u64 sort)
+#endif
+  static constexpr bool kStage = GSS_SCATTER_STAGE && (!kHasVal<Val> || sizeof(Key) + sizeof(Val) <= 8);
   static size_t bytes(uint32_t kmax) {
     size_t b = (size_t)kmax * 4 * 3;                            // cnt/off, delta, gbase
     b = (b + 15) & ~size_t(15);
-    b += (size_t)kChunk * sizeof(Key);
-    if (kHasVal<Val>) b += (size_t)kChunk * sizeof(Val);
+    b += (size_t)kChunk * sizeof(Key) * (kStage ? 2 : 1);
+    if (kHasVal<Val>) b += (size_t)kChunk * sizeof(Val) * (kStage ? 2 : 1);
     b += (size_t)kChunk * sizeof(IdT);
     return b;
   }
 };
 
 template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kScatterThreads, 2)
+__global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     k_scatter_fast(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
+  constexpr bool STAGE = ScatterFastSmem<Key, Val, IdT>::kStage;
   uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw);          // chunk counts, then run offsets
   uint32_t* delta = cnt + kmax;
   uint32_t* gbase = delta + kmax;
@@ -709,6 +722,10 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
   o += (size_t)kChunk * sizeof(Key);
   Val* svals = reinterpret_cast<Val*>(smem_raw + o);
   if constexpr (kHasVal<Val>) o += (size_t)kChunk * sizeof(Val);
+  Key* tkeys = reinterpret_cast<Key*>(smem_raw + o);              // staging (natural order)
+  if constexpr (STAGE) o += (size_t)kChunk * sizeof(Key);
+  Val* tvals = reinterpret_cast<Val*>(smem_raw + o);
+  if constexpr (STAGE && kHasVal<Val>) o += (size_t)kChunk * sizeof(Val);
   IdT* sids = reinterpret_cast<IdT*>(smem_raw + o);
 
   const uint32_t slot = level & 1;
@@ -728,30 +745,31 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
   const uint32_t t_end = min(nt, t + per);
   if (t >= t_end) return;
 
-  uint32_t beg, len, K, hrow, hstride, tl, blo, idb;
+  // per-tile state kept in registers: start, length, id base, K (the
+  // histogram row is re-read from the bucket record when a tile starts)
+  uint32_t beg, len, K, idb;
   auto tile_info = [&](uint32_t tt) {
-    const uint32_t b = c.tile_bucket[slot][tt];
-    const Bucket B = c.bk[slot][b];
-    tl = tt - B.tile_start;
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t tl = tt - B.tile_start;
     beg = B.lo + tl * c.T;
     len = min(c.T, B.m - tl * c.T);
     K = B.K;
-    hrow = B.hist_base;
-    hstride = B.ntiles;
-    blo = B.lo;
     idb = B.id_base + tl * c.T;
   };
-  auto load_gbase = [&]() {
-    const uint32_t* hist = c.hist[slot] + hrow;
+  auto load_gbase = [&](uint32_t tt) {
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t tl = tt - B.tile_start;
+    const uint32_t* hist = c.hist[slot] + B.hist_base;
     const uint32_t hb = hist[0];
-    for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
+    for (uint32_t id = threadIdx.x; id < B.K; id += kScatterThreads)
+      gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
   };
   tile_info(t);
-  load_gbase();
+  load_gbase(t);
   for (uint32_t id = threadIdx.x; id < kmax; id += kScatterThreads) cnt[id] = 0;
   Key pk[kScatterIter];
   Val pv[kScatterIter];
-  uint32_t pid[kScatterIter];
+  uint32_t pid[kScatterIter];                                      // id, or 0xffffffff past the chunk end
   auto load_chunk = [&](uint32_t cbeg, uint32_t cid, uint32_t clen) {
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
@@ -769,30 +787,58 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
   __syncthreads();                                                 // gbase and counters initialised
   for (;;) {
     const uint32_t clen = min((uint32_t)kChunk, len - c0);
+    uint32_t ir[kScatterIter];                                     // (rank << 16) | id; 0xffffffff = none
     Key kk[kScatterIter];
     Val vv[kScatterIter];
-    uint32_t iid[kScatterIter], rk[kScatterIter];
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
-      kk[it] = pk[it];
-      iid[it] = pid[it];
-      if constexpr (kHasVal<Val>) vv[it] = pv[it];
+      ir[it] = pid[it];
+      if constexpr (STAGE) {
+        // the keys (and values) wait in shared memory in natural order
+        if (ir[it] != 0xffffffffu) {
+          tkeys[q0 + it * 32] = pk[it];
+          if constexpr (kHasVal<Val>) tvals[q0 + it * 32] = pv[it];
+        }
+      } else {
+        kk[it] = pk[it];
+        if constexpr (kHasVal<Val>) vv[it] = pv[it];
+      }
     }
     // 1. rank within (chunk, id): one shared atomic per key on the CTA's counter
 #pragma unroll
-    for (int it = 0; it < kScatterIter; it++)
-      rk[it] = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, cnt_s + 4 * (iid[it] & 0xffffu), 1u);
+    for (int it = 0; it < kScatterIter; it++) {
+      const uint32_t id = ir[it] & 0xffffu;
+      const uint32_t r = atom_add_shared_if(ir[it] != 0xffffffffu ? 1u : 0u, cnt_s + 4 * id, 1u);
+      ir[it] = ir[it] == 0xffffffffu ? ir[it] : (r << 16) | id;
+    }
+    // advance and, with staging, prefetch the next chunk now: its loads
+    // overlap the scan, the reorder and the write-out of this one
+    const uint32_t cur_clen = clen, cur_K = K;
+#ifdef GSS_EXP_SEQWRITE
+    const uint32_t cur_beg = beg + c0;
+#endif
+    bool new_tile = false, done = false;
+    c0 += kChunk;
+    if (c0 >= len) {
+      t++;
+      c0 = 0;
+      if (t >= t_end) done = true;
+      else { tile_info(t); new_tile = true; }
+    }
+    if constexpr (STAGE) {
+      if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
+    }
     __syncthreads();
     // 2. warp 0: exclusive scan of the K chunk totals -> staged run offsets
     //    (cnt), staged -> global displacement (delta); gbase advances
     if (w == 0) {
       uint32_t run = 0;
-      for (uint32_t id0 = 0; id0 < K; id0 += 32 * 8) {
+      for (uint32_t id0 = 0; id0 < cur_K; id0 += 32 * 8) {
         const uint32_t ib = id0 + lane * 8;
         uint32_t x[8], sum = 0;
 #pragma unroll
         for (int j = 0; j < 8; j++) {
-          x[j] = ib + j < K ? cnt[ib + j] : 0u;
+          x[j] = ib + j < cur_K ? cnt[ib + j] : 0u;
           sum += x[j];
         }
         uint32_t inc = sum;
@@ -804,7 +850,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
         uint32_t ex = run + inc - sum;
 #pragma unroll
         for (int j = 0; j < 8; j++) {
-          if (ib + j < K) {
+          if (ib + j < cur_K) {
             cnt[ib + j] = ex;
             delta[ib + j] = gbase[ib + j] - ex;
             gbase[ib + j] += x[j];
@@ -818,38 +864,40 @@ __global__ void __launch_bounds__(kScatterThreads, 2)
     // 3. reorder the chunk by id in shared memory
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
-      if (iid[it] != 0xffffffffu) {
-        const uint32_t pos = cnt[iid[it]] + rk[it];
-        skeys[pos] = kk[it];
-        if constexpr (kHasVal<Val>) svals[pos] = vv[it];
-        sids[pos] = (IdT)iid[it];
+      if (ir[it] != 0xffffffffu) {
+        const uint32_t id = ir[it] & 0xffffu;
+        const uint32_t pos = cnt[id] + (ir[it] >> 16);
+        if constexpr (STAGE) {
+          skeys[pos] = tkeys[q0 + it * 32];
+          if constexpr (kHasVal<Val>) svals[pos] = tvals[q0 + it * 32];
+        } else {
+          skeys[pos] = kk[it];
+          if constexpr (kHasVal<Val>) svals[pos] = vv[it];
+        }
+        sids[pos] = (IdT)id;
       }
     }
-    // advance and prefetch the next chunk (possibly of the next tile)
-    const uint32_t cur_clen = clen, cur_K = K;
-    bool new_tile = false, done = false;
-    c0 += kChunk;
-    if (c0 >= len) {
-      t++;
-      c0 = 0;
-      if (t >= t_end) done = true;
-      else { tile_info(t); new_tile = true; }
+    if constexpr (!STAGE) {
+      if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
     }
-    if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
     __syncthreads();
     // 4. write this chunk's bucket runs; clear the counters for the next chunk
 #pragma unroll 4
     for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
+#ifdef GSS_EXP_SEQWRITE
+      const uint32_t d = cur_beg + q;                              // diagnostic: plain copy (wrong result)
+#else
       const uint32_t d = delta[sids[q]] + q;
+#endif
       kdst[d] = skeys[q];
       if constexpr (kHasVal<Val>) vdst[d] = svals[q];
     }
     for (uint32_t id = threadIdx.x; id < cur_K; id += kScatterThreads) cnt[id] = 0;
     if (done) break;
     if (new_tile) {
-      // gbase is rewritten only after every thread has left step 4
+      // gbase is rewritten only after every thread has left steps 2-4
       __syncthreads();
-      load_gbase();
+      load_gbase(t);
     }
     __syncthreads();
   }
