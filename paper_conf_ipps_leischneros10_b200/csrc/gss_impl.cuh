@@ -34,7 +34,7 @@ struct gss_profiler {
 namespace gssh {
 
 inline constexpr uint32_t kVersion = 1;
-inline constexpr uint32_t kFlagScatterWarpCounters = 1u << 30;   // ablation: unstable ranks from per-warp counters (k_scatter)
+inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -306,7 +306,7 @@ struct Engine {
     const size_t sm_sample = CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
     auto kc = k_classify<Key, Val, IdT, Cmp>;
     const size_t sm_cls = cls_smem_bytes<Key>(kmax);
-    auto ksc = k_scatter<Key, Val, IdT, Cmp>;
+    auto ksc = c.stable ? k_scatter<Key, Val, IdT, Cmp, true> : k_scatter<Key, Val, IdT, Cmp, false>;
     const size_t sm_sc = ScatterSmem<Key, Val, IdT>::bytes(kmax);
     GSS_TRY(set_smem(ks, sm_sample));
     GSS_TRY(set_smem(kc, sm_cls));
@@ -335,11 +335,12 @@ struct Engine {
                      [&] { k_scan_reduce<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
       GSS_TRY(launch(prof, GSS_K_SCAN, s, count,
                      [&] { k_scan_final<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
-      // stable ranks (R7 probe, GSS_FLAG_STABLE) and the per-warp-counter ablation: k_scatter;
-      // default: k_scatter_fast (one counter set per CTA); the paper's direct scatter: k_scatter_direct
-      if (c.stable || (cfg.flags & kFlagScatterWarpCounters)) {
+      // default and stable ranks (R7, GSS_FLAG_STABLE): k_scatter with per-warp counters (deterministic);
+      // ablations: k_scatter_fast (one counter set per CTA: atomic order across warps is not
+      // deterministic) and the paper's direct scatter (k_scatter_direct)
+      if (c.stable || !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters))) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));
-      } else if (!(cfg.flags & GSS_FLAG_DIRECT_SCATTER)) {
+      } else if (cfg.flags & kFlagScatterCtaCounters) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksf<<<g_sf, kScatterThreads, sm_sf, s>>>(c, l, kmax); }));
       } else {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count,

@@ -483,7 +483,7 @@ __device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t s
 // ...) chunk by chunk; the keys, values and ids of the next chunk are loaded
 // into registers before the current chunk's runs are written out, so the
 // global-load latency overlaps the write phase and the barriers.
-template <class Key, class Val, class IdT, class Cmp>
+template <class Key, class Val, class IdT, class Cmp, bool STABLE>
 __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   constexpr int NW = kScatterThreads / 32;
@@ -510,35 +510,33 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
   const IdT* idsrc = c.ids;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   const uint32_t ltmask = lanemask_lt();
-  const bool stable = c.stable != 0;
   uint32_t* wc = wcnt + w * kmax;
   const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
   const uint32_t q0 = w * (32 * kScatterIter) + lane;
 
   uint32_t t = blockIdx.x;
   if (t >= nt) return;
-  // tile state
-  uint32_t idb = 0;
-  auto tile_info = [&](uint32_t tt, uint32_t& beg, uint32_t& len, uint32_t& K, uint32_t& hrow, uint32_t& hstride,
-                       uint32_t& tl, uint32_t& lo) {
-    const uint32_t b = c.tile_bucket[slot][tt];
-    const Bucket B = c.bk[slot][b];
-    tl = tt - B.tile_start;
+  // per-tile state kept in registers: start, length, id base, K (the
+  // histogram row is re-read from the bucket record when a tile starts)
+  uint32_t beg, len, K, idb;
+  auto tile_info = [&](uint32_t tt) {
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t tl = tt - B.tile_start;
     beg = B.lo + tl * c.T;
     len = min(c.T, B.m - tl * c.T);
     K = B.K;
-    hrow = B.hist_base;
-    hstride = B.ntiles;
-    lo = B.lo;
     idb = B.id_base + tl * c.T;
   };
-  uint32_t beg, len, K, hrow, hstride, tl, blo;
-  tile_info(t, beg, len, K, hrow, hstride, tl, blo);
-  {
-    const uint32_t* hist = c.hist[slot] + hrow;
+  auto load_gbase = [&](uint32_t tt) {
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t tl = tt - B.tile_start;
+    const uint32_t* hist = c.hist[slot] + B.hist_base;
     const uint32_t hb = hist[0];
-    for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
-  }
+    for (uint32_t id = threadIdx.x; id < B.K; id += kScatterThreads)
+      gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
+  };
+  tile_info(t);
+  load_gbase(t);
   // prefetch registers: the chunk to process next
   Key pk[kScatterIter];
   Val pv[kScatterIter];
@@ -561,7 +559,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     const uint32_t clen = min((uint32_t)kChunk, len - c0);
     Key kk[kScatterIter];
     Val vv[kScatterIter];
-    uint32_t iid[kScatterIter], rk[kScatterIter];
+    uint32_t iid[kScatterIter];                                    // id; after ranking (rank << 16) | id
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
       kk[it] = pk[it];
@@ -570,7 +568,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     }
     for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
     __syncwarp();
-    if (stable) {
+    if constexpr (STABLE) {
       // Stable ranks (R7): peer masks of lanes holding the same bucket id, one
       // ballot per id bit; the lowest lane of each group adds the group size to
       // the warp's counter, so ranks follow lane order.
@@ -595,15 +593,19 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
         __syncwarp();
       }
 #pragma unroll
-      for (int it = 0; it < kScatterIter; it++)
-        rk[it] = __popc(peers[it] & ltmask) + __shfl_sync(kFull, old[it], __ffs(peers[it]) - 1);
+      for (int it = 0; it < kScatterIter; it++) {
+        const uint32_t r = __popc(peers[it] & ltmask) + __shfl_sync(kFull, old[it], __ffs(peers[it]) - 1);
+        iid[it] = iid[it] == 0xffffffffu ? iid[it] : (r << 16) | iid[it];
+      }
     } else {
       // One shared-memory atomic per key on the warp's own counters: ranks are
       // unique within (warp, id) in any order, so the level is a partition
       // whose within-bucket order is the hardware's atomic order.
 #pragma unroll
-      for (int it = 0; it < kScatterIter; it++)
-        rk[it] = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (iid[it] & 0xffffu), 1u);
+      for (int it = 0; it < kScatterIter; it++) {
+        const uint32_t r = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (iid[it] & 0xffffu), 1u);
+        iid[it] = iid[it] == 0xffffffffu ? iid[it] : (r << 16) | iid[it];
+      }
     }
     __syncthreads();
     // chunk totals per id, exclusive scan over ids, then every warp's start
@@ -643,10 +645,11 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
       if (iid[it] != 0xffffffffu) {
-        const uint32_t pos = wc[iid[it]] + rk[it];
+        const uint32_t id = iid[it] & 0xffffu;
+        const uint32_t pos = wc[id] + (iid[it] >> 16);
         skeys[pos] = kk[it];
         if constexpr (kHasVal<Val>) svals[pos] = vv[it];
-        sids[pos] = (IdT)iid[it];
+        sids[pos] = (IdT)id;
       }
     }
     __syncthreads();
@@ -660,7 +663,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       c0 = 0;
       if (t >= nt) done = true;
       else {
-        tile_info(t, beg, len, K, hrow, hstride, tl, blo);
+        tile_info(t);
         new_tile = true;
       }
     }
@@ -674,11 +677,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     }
     __syncthreads();
     if (done) break;
-    if (new_tile) {
-      const uint32_t* hist = c.hist[slot] + hrow;
-      const uint32_t hb = hist[0];
-      for (uint32_t id = threadIdx.x; id < K; id += kScatterThreads) gbase[id] = hist[id * hstride + tl] - hb + blo;
-    }
+    if (new_tile) load_gbase(t);
   }
 }
 
