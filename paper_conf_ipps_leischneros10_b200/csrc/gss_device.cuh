@@ -11,13 +11,16 @@
 
 namespace gss {
 
-// In-SM sort size classes (R8): class i holds buckets sorted by a CTA of
-// class_warps(i) warps, i.e. up to class_warps(i) * 32 * sort_items keys
-// (1..16 warps one by one, then 20, 24, 28, 32).  Fine classes keep every
-// thread of a bucket's CTA busy: with power-of-two classes a bucket just
-// above a class boundary left half of its CTA idle at every merge barrier.
-constexpr int kNumClasses = 20;
-__host__ __device__ constexpr int class_warps(int i) { return i < 16 ? i + 1 : 16 + 4 * (i - 15); }
+// In-SM sort size classes (R8): class i holds the buckets sorted by a CTA of
+// class_warps(i) warps, i.e. up to class_warps(i) * 32 * sort_items keys:
+// 1..8 warps one by one, then 10, 12, 16, 24, 32.  Fine classes keep most
+// threads of a bucket's CTA busy (with power-of-two classes a bucket just
+// above a class boundary left half of its CTA idle at every merge barrier);
+// few enough that the empty ones cost little in launch-bound sorts.
+constexpr int kNumClasses = 13;
+__host__ __device__ constexpr int class_warps(int i) {
+  return i < 8 ? i + 1 : (i == 8 ? 10 : (i == 9 ? 12 : (i == 10 ? 16 : (i == 11 ? 24 : 32))));
+}
 constexpr int kMaxLevels = 16;        // distribution levels launched at most
 constexpr uint32_t kFull = 0xffffffffu;
 

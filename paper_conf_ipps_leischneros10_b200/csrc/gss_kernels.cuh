@@ -21,8 +21,14 @@ constexpr int kClsThreads = 256;
 #ifndef GSS_SCATTER_MINB
 #define GSS_SCATTER_MINB 2
 #endif
+#ifndef GSS_SCATTER_EARLY
+#define GSS_SCATTER_EARLY 0
+#endif
 constexpr int kScatterThreads = GSS_SCATTER_THREADS;
-constexpr int kScatterIter = 8;                                   // keys per thread per chunk
+#ifndef GSS_SCATTER_ITER
+#define GSS_SCATTER_ITER 8
+#endif
+constexpr int kScatterIter = GSS_SCATTER_ITER;                      // keys per thread per chunk
 constexpr int kChunk = kScatterThreads * kScatterIter;            // 4096 keys staged per chunk
 constexpr int kScanCtas = 256;
 constexpr int kScanThreads = 256;
@@ -566,7 +572,24 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       iid[it] = pid[it];
       if constexpr (kHasVal<Val>) vv[it] = pv[it];
     }
-    for (uint32_t id = lane; id < K; id += 32) wc[id] = 0;
+    const uint32_t cur_K = K, cur_clen = clen;
+    bool new_tile = false;
+    bool done = false;
+#if GSS_SCATTER_EARLY
+    // advance and prefetch the next chunk at once: its loads overlap this whole chunk
+    c0 += kChunk;
+    if (c0 >= len) {
+      t += gridDim.x;
+      c0 = 0;
+      if (t >= nt) done = true;
+      else {
+        tile_info(t);
+        new_tile = true;
+      }
+    }
+    if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
+#endif
+    for (uint32_t id = lane; id < cur_K; id += 32) wc[id] = 0;
     __syncwarp();
     if constexpr (STABLE) {
       // Stable ranks (R7): peer masks of lanes holding the same bucket id, one
@@ -611,12 +634,12 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     // chunk totals per id, exclusive scan over ids, then every warp's start
     // within each id folded into its counter (one lookup per key below)
     {
-      const uint32_t per = (K + kScatterThreads - 1) / kScatterThreads;
+      const uint32_t per = (cur_K + kScatterThreads - 1) / kScatterThreads;
       const uint32_t i0 = threadIdx.x * per;
       uint32_t tsum = 0;
       for (uint32_t j = 0; j < per; j++) {
         const uint32_t id = i0 + j;
-        if (id < K) {
+        if (id < cur_K) {
           uint32_t tt = 0;
 #pragma unroll
           for (int q = 0; q < NW; q++) tt += wcnt[q * kmax + id];
@@ -627,7 +650,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       uint32_t ex = block_exclusive_scan<kScatterThreads>(tsum, s_warp, nullptr);
       for (uint32_t j = 0; j < per; j++) {
         const uint32_t id = i0 + j;
-        if (id < K) {
+        if (id < cur_K) {
           uint32_t run = ex;
 #pragma unroll
           for (int q = 0; q < NW; q++) {
@@ -653,10 +676,8 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       }
     }
     __syncthreads();
+#if !GSS_SCATTER_EARLY
     // advance and prefetch the next chunk (possibly of the next tile)
-    const uint32_t cur_clen = clen;
-    bool new_tile = false;
-    bool done = false;
     c0 += kChunk;
     if (c0 >= len) {
       t += gridDim.x;
@@ -668,6 +689,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       }
     }
     if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
+#endif
     // write this chunk's bucket runs
 #pragma unroll 4
     for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
