@@ -294,6 +294,36 @@ __device__ __forceinline__ void oem_sort(Key* k, Val* v, Cmp less) {
   }
 }
 
+// Bitonic sort network on k[0 .. N) (N a power of two), compile-time indices:
+// the alternative the paper measured against odd-even merge;
+// selected with -DGSS_THREAD_NET=1 (ablation).
+template <int N, class Key, class Val, class Cmp>
+__device__ __forceinline__ void bitonic_sort_regs(Key* k, Val* v, Cmp less) {
+#pragma unroll
+  for (int size = 2; size <= N; size <<= 1) {
+#pragma unroll
+    for (int stride = size >> 1; stride > 0; stride >>= 1) {
+#pragma unroll
+      for (int i = 0; i < N; i++) {
+        const int j = i ^ stride;
+        if (j > i) {
+          if ((i & size) == 0) cmp_swap(k[i], k[j], v[i], v[j], less);
+          else cmp_swap(k[j], k[i], v[j], v[i], less);
+        }
+      }
+    }
+  }
+}
+
+#ifndef GSS_THREAD_NET
+#define GSS_THREAD_NET 0   // 0: Batcher odd-even merge sort (default), 1: bitonic sort
+#endif
+template <int N, class Key, class Val, class Cmp>
+__device__ __forceinline__ void thread_sort_net(Key* k, Val* v, Cmp less) {
+  if constexpr (GSS_THREAD_NET == 1) bitonic_sort_regs<N>(k, v, less);
+  else oem_sort<0, N>(k, v, less);
+}
+
 // Stable odd-even transposition sort (only for the one partial thread).
 template <int N, class Key, class Val, class Cmp>
 __device__ __forceinline__ void transposition_sort(Key* k, Val* v, Cmp less) {
@@ -541,9 +571,9 @@ struct CtaSort {
       }
       if constexpr (KV) {
         if (stable_path) transposition_sort<ITEMS>(k, v, less);
-        else oem_sort<0, ITEMS>(k, v, less);
+        else thread_sort_net<ITEMS>(k, v, less);
       } else {
-        oem_sort<0, ITEMS>(k, v, less);
+        thread_sort_net<ITEMS>(k, v, less);
       }
     }
     __syncwarp();

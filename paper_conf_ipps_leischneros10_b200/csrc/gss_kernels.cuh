@@ -276,7 +276,10 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
                                               uint32_t len, uint32_t tree_s, uint32_t rep_b, const Key* spl,
                                               uint32_t logk, uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid,
                                               Cmp less) {
-  constexpr int U = 8;
+#ifndef GSS_CLS_U
+#define GSS_CLS_U 8
+#endif
+  constexpr int U = GSS_CLS_U;                                 // keys per lane per group
   constexpr uint32_t G = U * kClsThreads;                      // keys per group
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   const uint32_t off = (uint32_t)w * (32 * U) + lane;
@@ -305,9 +308,12 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
     __syncwarp();
     // lane l writes ids [l*U, l*U + U) of the warp's 256 (U * sizeof(IdT) bytes)
     IdT* gp = tids + g * G + (uint32_t)w * (32 * U) + lane * U;
-    if constexpr (sizeof(IdT) == 1) {
+    if constexpr (U * sizeof(IdT) == 4) {
+      *reinterpret_cast<uint32_t*>(gp) = *reinterpret_cast<const uint32_t*>(wid + lane * U);
+    } else if constexpr (U * sizeof(IdT) == 8) {
       *reinterpret_cast<uint2*>(gp) = *reinterpret_cast<const uint2*>(wid + lane * U);
     } else {
+      static_assert(U * sizeof(IdT) == 16, "ids per lane: 4, 8 or 16 bytes");
       *reinterpret_cast<uint4*>(gp) = *reinterpret_cast<const uint4*>(wid + lane * U);
     }
     __syncwarp();
