@@ -101,8 +101,9 @@ typedef struct gss_params {
   gss_profiler* profiler;   /* optional: CUDA-event time of every launch                   */
 } gss_params;
 
-#define GSS_FLAG_RECOMPUTE_IDS 1u  /* Phase 4 re-descends the tree instead of reading stored
-                                      bucket ids (the paper's choice); reserved  */
+#define GSS_FLAG_RECOMPUTE_IDS 1u  /* Phase 4 re-descends the splitter tree instead of reading
+                                      bucket ids stored by Phase 2 (the paper's choice,
+                                      P:264-267; ablation: slower on B200); sorts only       */
 #define GSS_FLAG_STABLE 4u         /* Phase 4 ranks keys stably (R7: each level is a stable
                                       partition); default: one shared atomic per key, which
                                       partitions correctly but orders keys within a bucket in

@@ -94,7 +94,6 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   c->fill_div = p.fill_div ? p.fill_div : 4;
   c->seed = p.seed ? p.seed : 5489;
   c->flags = p.flags;
-  if (c->flags & GSS_FLAG_RECOMPUTE_IDS) return GSS_ERROR_NOT_SUPPORTED;
   // size classes (R8): class i = buckets a CTA of class_warps(i) warps sorts
   c->nclass = kNumClasses;
   for (int i = 0; i < kNumClasses; i++) c->class_cap[i] = (uint32_t)(class_warps(i) * 32 * small_items<Key, Val>());
@@ -262,6 +261,8 @@ struct Engine {
     c.L = mode == MODE_SORT ? cfg.L : 1;
     c.mode = mode;
     c.stable = ((cfg.flags & GSS_FLAG_STABLE) || mode != MODE_SORT) ? 1u : 0u;   // partitions stay stable (R7 probe)
+    c.recompute = (!c.stable && (cfg.flags & GSS_FLAG_RECOMPUTE_IDS) && !(cfg.flags & GSS_FLAG_DIRECT_SCATTER) &&
+                   !(cfg.flags & kFlagScatterCtaCounters)) ? 1u : 0u;
     c.cap_buckets = lay.cap_buckets; c.cap_tiles = lay.cap_tiles; c.cap_hist = lay.cap_hist;
     c.cap_spl = lay.cap_spl; c.cap_copy = lay.cap_copy; c.cap_ovf = lay.cap_ovf;
     c.cap_fb = lay.cap_fb;
@@ -306,8 +307,9 @@ struct Engine {
     const size_t sm_sample = CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
     auto kc = k_classify<Key, Val, IdT, Cmp>;
     const size_t sm_cls = cls_smem_bytes<Key>(kmax);
-    auto ksc = c.stable ? k_scatter<Key, Val, IdT, Cmp, true> : k_scatter<Key, Val, IdT, Cmp, false>;
-    const size_t sm_sc = ScatterSmem<Key, Val, IdT>::bytes(kmax);
+    auto ksc = c.stable ? k_scatter<Key, Val, IdT, Cmp, true>
+                        : (c.recompute ? k_scatter<Key, Val, IdT, Cmp, false, true> : k_scatter<Key, Val, IdT, Cmp, false>);
+    const size_t sm_sc = ScatterSmem<Key, Val, IdT>::bytes(kmax, c.recompute != 0);
     GSS_TRY(set_smem(ks, sm_sample));
     GSS_TRY(set_smem(kc, sm_cls));
     GSS_TRY(set_smem(ksc, sm_sc));

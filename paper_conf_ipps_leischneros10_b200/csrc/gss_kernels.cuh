@@ -271,7 +271,7 @@ __device__ __forceinline__ void descend_group(const Key (&e)[U], uint32_t (&id)[
 // the warp stages its 256 ids in shared memory and writes them as one 8-byte
 // store per lane.  Full groups run without bounds tests; the next group's
 // keys are loaded before this group descends.
-template <int MODE, class Key, class IdT, class Cmp>
+template <int MODE, bool STORE, class Key, class IdT, class Cmp>
 __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* __restrict__ tids, uint32_t beg,
                                               uint32_t len, uint32_t tree_s, uint32_t rep_b, const Key* spl,
                                               uint32_t logk, uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid,
@@ -303,8 +303,9 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
 #pragma unroll
     for (int u = 0; u < U; u++) {
       red_shared_add(wc_s + 4 * id[u], 1u);
-      wid[u * 32 + lane] = (IdT)id[u];
+      if constexpr (STORE) wid[u * 32 + lane] = (IdT)id[u];
     }
+    if constexpr (!STORE) continue;                            // GSS_FLAG_RECOMPUTE_IDS: Phase 4 re-descends
     __syncwarp();
     // lane l writes ids [l*U, l*U + U) of the warp's 256 (U * sizeof(IdT) bytes)
     IdT* gp = tids + g * G + (uint32_t)w * (32 * U) + lane * U;
@@ -335,7 +336,7 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
       const uint32_t i = tb + off + u * 32;
       if (i < len) {
         red_shared_add(wc_s + 4 * id[u], 1u);
-        tids[i] = (IdT)id[u];
+        if constexpr (STORE) tids[i] = (IdT)id[u];
       }
     }
   }
@@ -391,9 +392,16 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
     const uint32_t len = min(c.T, B.m - tl * c.T);
     const uint32_t logk = ilog2(B.ks);
     IdT* tids = c.ids + B.id_base + tl * c.T;                  // 16-byte aligned per tile
-    if (B.eq) classify_tile<1>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
-    else if (B.clamp) classify_tile<2>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
-    else classify_tile<0>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    if (c.recompute) {
+      if (B.eq) classify_tile<1, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+      else classify_tile<0, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    } else if (B.eq) {
+      classify_tile<1, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    } else if (B.clamp) {
+      classify_tile<2, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    } else {
+      classify_tile<0, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    }
     __syncthreads();
     uint32_t* hist = c.hist[slot] + B.hist_base;
     for (uint32_t id = threadIdx.x; id < B.K; id += kClsThreads) {
@@ -467,8 +475,13 @@ __global__ void __launch_bounds__(kScanThreads) k_scan_final(Ctx<Key, Val, IdT> 
 // ---------------------------------------------------------------------------
 template <class Key, class Val, class IdT>
 struct ScatterSmem {
-  static size_t bytes(uint32_t kmax) {
-    size_t b = 0;
+  // splitter tree, sorted splitters and bank-replicated middle levels, as in
+  // k_classify (only with GSS_FLAG_RECOMPUTE_IDS)
+  __host__ __device__ static size_t tree_bytes(uint32_t kmax) {
+    return (size_t)kmax * sizeof(Key) * 2 + (size_t)kRepNodes * 128;
+  }
+  static size_t bytes(uint32_t kmax, bool recompute = false) {
+    size_t b = recompute ? tree_bytes(kmax) : 0;
     b += (size_t)kmax * 4 * 3;                                  // gbase, ctot, delta
     b += (size_t)(kScatterThreads / 32) * kmax * 4;             // per-warp counters
     b += 64;                                                    // scan scratch
@@ -495,21 +508,33 @@ __device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t s
 // ...) chunk by chunk; the keys, values and ids of the next chunk are loaded
 // into registers before the current chunk's runs are written out, so the
 // global-load latency overlaps the write phase and the barriers.
-template <class Key, class Val, class IdT, class Cmp, bool STABLE>
+// RECOMP (GSS_FLAG_RECOMPUTE_IDS, the paper's choice): no stored
+// ids; every key re-descends its bucket's splitter tree (same layout and
+// descent as k_classify) when its chunk is ranked.
+template <class Key, class Val, class IdT, class Cmp, bool STABLE, bool RECOMP = false>
 __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   constexpr int NW = kScatterThreads / 32;
-  uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);
+  constexpr uint32_t REP = rep_copies<Key>();
+  Key* tree = reinterpret_cast<Key*>(smem_raw);
+  Key* spl = tree + kmax;
+  Key* rep = spl + kmax;
+  const size_t tb = RECOMP ? ScatterSmem<Key, Val, IdT>::tree_bytes(kmax) : 0;
+  const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
+  const uint32_t rep_b = (uint32_t)__cvta_generic_to_shared(rep) - (1u << kTopLevels) * 128u +
+                         (threadIdx.x % REP) * (uint32_t)sizeof(Key);
+  uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw + tb);
   uint32_t* ctot = gbase + kmax;
   uint32_t* delta = ctot + kmax;
   uint32_t* wcnt = delta + kmax;
   uint32_t* s_warp = wcnt + NW * kmax;
-  size_t off = ((size_t)(kmax * 3 + NW * kmax) * 4 + 64 + 15) & ~size_t(15);
+  size_t off = tb + (((size_t)(kmax * 3 + NW * kmax) * 4 + 64 + 15) & ~size_t(15));
   Key* skeys = reinterpret_cast<Key*>(smem_raw + off);
   off += (size_t)kChunk * sizeof(Key);
   Val* svals = reinterpret_cast<Val*>(smem_raw + off);
   if constexpr (kHasVal<Val>) off += (size_t)kChunk * sizeof(Val);
   IdT* sids = reinterpret_cast<IdT*>(smem_raw + off);
+  const Cmp less;
 
   const uint32_t slot = level & 1;
   const uint32_t nt = c.cnt->lvl[level].num_tiles;
@@ -531,13 +556,30 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
   // per-tile state kept in registers: start, length, id base, K (the
   // histogram row is re-read from the bucket record when a tile starts)
   uint32_t beg, len, K, idb;
+  uint32_t tmode = 0, tks = 0, cur_b = 0xffffffffu, next_b = 0;   // RECOMP: id rule and tree of the tile's bucket
   auto tile_info = [&](uint32_t tt) {
-    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t bi = c.tile_bucket[slot][tt];
+    const Bucket B = c.bk[slot][bi];
     const uint32_t tl = tt - B.tile_start;
     beg = B.lo + tl * c.T;
     len = min(c.T, B.m - tl * c.T);
     K = B.K;
     idb = B.id_base + tl * c.T;
+    next_b = bi;
+  };
+  // RECOMP: the tile's tree into shared memory (a barrier must precede and follow)
+  auto load_tree = [&](uint32_t bi) {
+    const Bucket B = c.bk[slot][bi];
+    const Key* g = c.spl[slot] + B.spl_base;
+    for (uint32_t j = threadIdx.x + 1; j < B.ks; j += kScatterThreads) tree[j] = g[j];
+    for (uint32_t j = threadIdx.x; j + 1 < B.ks; j += kScatterThreads) spl[j] = g[B.kb + j];
+    if (B.ks > (1u << kTopLevels)) {
+      const uint32_t nrep = (min(B.ks, 1u << kRepEnd) - (1u << kTopLevels)) * REP;
+      for (uint32_t q = threadIdx.x; q < nrep; q += kScatterThreads) rep[q] = g[(1u << kTopLevels) + q / REP];
+    }
+    tmode = B.eq ? 1u : (B.clamp ? 2u : 0u);
+    tks = B.ks;
+    cur_b = bi;
   };
   auto load_gbase = [&](uint32_t tt) {
     const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
@@ -549,6 +591,10 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
   };
   tile_info(t);
   load_gbase(t);
+  if constexpr (RECOMP) {
+    load_tree(next_b);
+    __syncthreads();
+  }
   // prefetch registers: the chunk to process next
   Key pk[kScatterIter];
   Val pv[kScatterIter];
@@ -560,7 +606,8 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       pid[it] = 0xffffffffu;
       if (q < clen) {
         pk[it] = ksrc[cbeg + q];
-        pid[it] = idsrc[cid + q];
+        if constexpr (RECOMP) pid[it] = 0u;                     // id computed when the chunk is ranked
+        else pid[it] = idsrc[cid + q];
         if constexpr (kHasVal<Val>) pv[it] = vsrc[cbeg + q];
       }
     }
@@ -577,6 +624,16 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       kk[it] = pk[it];
       iid[it] = pid[it];
       if constexpr (kHasVal<Val>) vv[it] = pv[it];
+    }
+    if constexpr (RECOMP) {
+      // re-descend (Algorithm 2) with the tile mode's id rule
+      uint32_t id[kScatterIter];
+      const uint32_t logk = ilog2(tks);
+      if (tmode == 1) descend_group<1>(kk, id, tree_s, rep_b, spl, logk, tks, K, less);
+      else if (tmode == 2) descend_group<2>(kk, id, tree_s, rep_b, spl, logk, tks, K, less);
+      else descend_group<0>(kk, id, tree_s, rep_b, spl, logk, tks, K, less);
+#pragma unroll
+      for (int it = 0; it < kScatterIter; it++) iid[it] = iid[it] == 0xffffffffu ? iid[it] : id[it];
     }
     const uint32_t cur_K = K, cur_clen = clen;
     bool new_tile = false;
@@ -705,7 +762,16 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     }
     __syncthreads();
     if (done) break;
-    if (new_tile) load_gbase(t);
+    if (new_tile) {
+      load_gbase(t);
+      if constexpr (RECOMP) {
+        if (next_b != cur_b) {
+          __syncthreads();                                     // every key of the old tile is ranked
+          load_tree(next_b);
+          __syncthreads();                                     // the new tree is complete before the next descent
+        }
+      }
+    }
   }
 }
 

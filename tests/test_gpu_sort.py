@@ -258,6 +258,36 @@ def test_single_bucket(gss, oracle_mod, width, pairs, m, flags):
             check_pairs(x, to_host(vo), want)
 
 
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist", ["uniform", "dd", "and3", "staggered"])
+def test_recompute_ids_ablation(gss, oracle_mod, width, pairs, dist):
+    """GSS_FLAG_RECOMPUTE_IDS (the paper's Phase 4: re-descend the tree
+    instead of reading stored ids) gives the oracle's keys through several levels."""
+    n = (1 << 20) + 999
+    x = inputs.keys(dist, n, width, seed=5)
+    v = inputs.values(n, width) if pairs else None
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=4096, flags=1, stats=True)
+    assert st.error_flags == 0 and st.levels >= 2
+    want = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=4096))[0]
+    np.testing.assert_array_equal(to_host(ko), want)
+    if pairs:
+        check_pairs(x, to_host(vo), want)
+
+
+def test_recompute_ids_ablation_large(gss, oracle_mod):
+    """GSS_FLAG_RECOMPUTE_IDS at 2^24 keys (hundreds of tiles per CTA, a tree
+    reload at every tile of level 1): sorted, same multiset, sampled ranks."""
+    n = 1 << 24
+    x = inputs.keys("uniform", n, 64, seed=6)
+    ko, _, st = gss.sort(to_dev(x), flags=1, stats=True)
+    assert st.error_flags == 0 and st.levels == 2
+    y = to_host(ko)
+    assert np.all(y[1:] >= y[:-1])
+    np.testing.assert_array_equal(np.sort(x[::4097]), np.sort(y[np.searchsorted(y, x[::4097])]))
+    for r in (0, n // 2, n - 1):
+        assert int(y[r]) == oracle_mod.select(x, r)
+
+
 def test_distributed_sorter_single_rank_nccl(gss):
     """The distributed path on one rank over NCCL: sample, sort, partition_by, all-to-all-v, sort."""
     import torch.distributed as dist
