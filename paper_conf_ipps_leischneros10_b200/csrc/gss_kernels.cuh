@@ -614,6 +614,13 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
   };
   uint32_t c0 = 0;
   load_chunk(beg, idb, min((uint32_t)kChunk, len));
+#ifdef GSS_SCATTER_PHASES
+  unsigned long long ph[6] = {0, 0, 0, 0, 0, 0}, tp = clock64();
+  uint32_t nchunks = 0;
+#define GSS_PH(i) do { const unsigned long long tn = clock64(); ph[i] += tn - tp; tp = tn; } while (0)
+#else
+#define GSS_PH(i) do {} while (0)
+#endif
   for (;;) {
     const uint32_t clen = min((uint32_t)kChunk, len - c0);
     Key kk[kScatterIter];
@@ -694,6 +701,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       }
     }
     __syncthreads();
+    GSS_PH(0);
     // chunk totals per id, exclusive scan over ids, then every warp's start
     // within each id folded into its counter (one lookup per key below)
     {
@@ -728,6 +736,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       }
     }
     __syncthreads();
+    GSS_PH(1);
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
       if (iid[it] != 0xffffffffu) {
@@ -739,6 +748,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       }
     }
     __syncthreads();
+    GSS_PH(2);
 #if !GSS_SCATTER_EARLY
     // advance and prefetch the next chunk (possibly of the next tile)
     c0 += kChunk;
@@ -761,6 +771,13 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       if constexpr (kHasVal<Val>) vdst[d] = svals[q];
     }
     __syncthreads();
+    GSS_PH(3);
+#ifdef GSS_SCATTER_PHASES
+    nchunks++;
+    if (done && threadIdx.x == 0 && (blockIdx.x == 0 || blockIdx.x == 100))
+      printf("scatter phases block %d chunks %u: rank %llu scan %llu reorder %llu write %llu (cycles per chunk)\n",
+             blockIdx.x, nchunks, ph[0] / nchunks, ph[1] / nchunks, ph[2] / nchunks, ph[3] / nchunks);
+#endif
     if (done) break;
     if (new_tile) {
       load_gbase(t);
@@ -878,6 +895,10 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   uint32_t c0 = 0;
   load_chunk(beg, idb, min((uint32_t)kChunk, len));
   __syncthreads();                                                 // gbase and counters initialised
+#ifdef GSS_SCATTER_PHASES
+  unsigned long long ph[6] = {0, 0, 0, 0, 0, 0}, tp = clock64();
+  uint32_t nchunks = 0;
+#endif
   for (;;) {
     const uint32_t clen = min((uint32_t)kChunk, len - c0);
     uint32_t ir[kScatterIter];                                     // (rank << 16) | id; 0xffffffff = none
@@ -922,6 +943,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
     }
     __syncthreads();
+    GSS_PH(0);
     // 2. warp 0: exclusive scan of the K chunk totals -> staged run offsets
     //    (cnt), staged -> global displacement (delta); gbase advances
     if (w == 0) {
@@ -954,6 +976,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       }
     }
     __syncthreads();
+    GSS_PH(1);
     // 3. reorder the chunk by id in shared memory
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
@@ -974,6 +997,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
     }
     __syncthreads();
+    GSS_PH(2);
     // 4. write this chunk's bucket runs; clear the counters for the next chunk
 #pragma unroll 4
     for (uint32_t q = threadIdx.x; q < cur_clen; q += kScatterThreads) {
@@ -986,6 +1010,13 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       if constexpr (kHasVal<Val>) vdst[d] = svals[q];
     }
     for (uint32_t id = threadIdx.x; id < cur_K; id += kScatterThreads) cnt[id] = 0;
+#ifdef GSS_SCATTER_PHASES
+    { const unsigned long long tn = clock64(); ph[3] += tn - tp; tp = tn; }
+    nchunks++;
+    if (done && threadIdx.x == 0 && (blockIdx.x == 0 || blockIdx.x == 100))
+      printf("fast scatter phases block %d chunks %u: rank %llu scan %llu reorder %llu write %llu (cycles per chunk)\n",
+             blockIdx.x, nchunks, ph[0] / nchunks, ph[1] / nchunks, ph[2] / nchunks, ph[3] / nchunks);
+#endif
     if (done) break;
     if (new_tile) {
       // gbase is rewritten only after every thread has left steps 2-4
