@@ -55,6 +55,15 @@ def peaks():
     return 6650.0, "fallback (B200_PROFILING.md: 6.65 TB/s)"
 
 
+def auto_k(n: int, M: int) -> int:
+    """The library's default k (gss.h, R29): 256, doubled while two levels would
+    leave final buckets above M/2 (2^30 u64 keys: 512)."""
+    k = 256
+    while k < 1024 and n > k * k * (M // 2):
+        k *= 2
+    return k
+
+
 def alg_bytes(kind: str, st, wk: int, wv: int, k: int, T: int, a: int, steps: int = 1) -> float:
     """Algorithmic bytes per step of one kernel kind."""
     split = sum(st.split_elems)
@@ -198,10 +207,10 @@ def run_ours(args, wl):
     wk = bits // 8
     wv = wk if pairs else 0
     kind = f"u{bits}"
-    params = dict(k=256, a=30, tile=32768, flags=16)            # flags 16: replay the launch sequence as a CUDA graph
+    M = 8192 if (pairs and bits == 64) else 16384
+    params = dict(k=auto_k(n, M), a=30, tile=65536, flags=16)   # flags 16: replay the launch sequence as a CUDA graph
     if wl == "c1_u32_2p16":
         params.update(k=128, k_policy="fixed")
-    M = 8192 if (pairs and bits == 64) else 16384
     params["M"] = M
 
     # input: this rank's shard of the global input (weak scaling: n keys per GPU)

@@ -86,7 +86,8 @@ typedef struct gss_profiler gss_profiler;
 /* Tuning and method parameters; pass NULL for the per-type defaults. A zero
  * field also selects its default. */
 typedef struct gss_params {
-  uint32_t k;               /* max buckets per split: power of 2 in [2,1024]      */
+  uint32_t k;               /* max buckets per split: power of 2 in [2,1024]; 0 ->
+                               256, or 512 / 1024 when n > k*k*M/2 (two levels suffice)  */
   uint32_t oversample;      /* a; 0 -> 30                               */
   uint64_t small_threshold; /* M: buckets with m <= M go to the in-SM sort;       */
                             /* 0 -> the in-SM capacity of the type; at most that           */

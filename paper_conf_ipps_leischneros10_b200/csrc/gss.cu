@@ -29,10 +29,10 @@ gss_status gss_default_params(uint32_t key_bytes, uint32_t val_bytes, gss_params
   if (!out || (key_bytes != 4 && key_bytes != 8) || (val_bytes != 0 && val_bytes != key_bytes))
     return GSS_ERROR_INVALID_VALUE;
   memset(out, 0, sizeof(*out));
-  out->k = 256;
+  out->k = 0;                                   // n-dependent: 256, or 512 / 1024 for large n (see gss.h)
   out->oversample = 30;
   out->small_threshold = (val_bytes && key_bytes + val_bytes > 8) ? 8192 : 16384;
-  out->tile = 32768;
+  out->tile = 65536;
   out->k_policy = 1;
   out->fill_div = 4;
   out->seed = 5489;
