@@ -207,7 +207,7 @@ def run_ours(args, wl):
     wk = bits // 8
     wv = wk if pairs else 0
     kind = f"u{bits}"
-    M = 8192 if (pairs and bits == 64) else 16384
+    M = 8192 if (pairs and bits == 64) else (32768 if (bits == 32 and not pairs) else 16384)   # in-SM capacity (R5)
     params = dict(k=auto_k(n, M), a=30, tile=65536, flags=16)   # flags 16: replay the launch sequence as a CUDA graph
     if wl == "c1_u32_2p16":
         params.update(k=128, k_policy="fixed")

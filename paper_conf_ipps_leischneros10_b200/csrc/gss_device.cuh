@@ -495,21 +495,29 @@ struct CtaSort {
   __device__ static __forceinline__ void store_run(Key* sk, Val* sv, const Key* k, const Val* v, int cnt, int rs,
                                                    int rlen, int o, bool desc) {
     // ascending: slots rs+o .. rs+o+ITEMS-1; descending: rs+rlen-o-ITEMS .. rs+rlen-o-1
-    if (ITEMS <= 16 && cnt == ITEMS && (((desc ? rs + rlen - o : rs + o)) & (ITEMS - 1)) == 0) {
-      // the ITEMS slots lie in one padded row of 16: consecutive addresses, immediate offsets
+    constexpr int RUN = ITEMS < 16 ? ITEMS : 16;                 // slots per padded row segment
+    if (cnt == ITEMS && (((desc ? rs + rlen - o : rs + o)) & (RUN - 1)) == 0) {
+      // the ITEMS slots fill whole padded rows (or lie in one): consecutive
+      // addresses per row, immediate offsets
       if (desc) {
-        const int q = phys(rs + rlen - 1 - o);
 #pragma unroll
-        for (int i = 0; i < ITEMS; i++) {
-          sk[q - i] = k[i];
-          if constexpr (KV) sv[q - i] = v[i];
+        for (int r = 0; r < ITEMS / RUN; r++) {
+          const int q = phys(rs + rlen - 1 - o - r * RUN);
+#pragma unroll
+          for (int i = 0; i < RUN; i++) {
+            sk[q - i] = k[r * RUN + i];
+            if constexpr (KV) sv[q - i] = v[r * RUN + i];
+          }
         }
       } else {
-        const int q = phys(rs + o);
 #pragma unroll
-        for (int i = 0; i < ITEMS; i++) {
-          sk[q + i] = k[i];
-          if constexpr (KV) sv[q + i] = v[i];
+        for (int r = 0; r < ITEMS / RUN; r++) {
+          const int q = phys(rs + o + r * RUN);
+#pragma unroll
+          for (int i = 0; i < RUN; i++) {
+            sk[q + i] = k[r * RUN + i];
+            if constexpr (KV) sv[q + i] = v[r * RUN + i];
+          }
         }
       }
       return;

@@ -74,7 +74,7 @@ struct Cfg {
 
 template <class Key, class Val>
 constexpr uint32_t max_small_capacity() {
-  return (kHasVal<Val> && sizeof(Key) + sizeof(Val) > 8) ? 8192u : 16384u;
+  return 32u * 32u * (uint32_t)small_items<Key, Val>();        // a 32-warp CTA
 }
 
 template <class Key, class Val>

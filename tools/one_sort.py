@@ -25,7 +25,7 @@ n, bits, pairs, dist, _ = bench.WORKLOADS[args.workload]
 x = inputs.keys(dist, n, bits, seed=1)
 k = torch.from_numpy(x).cuda()
 v = torch.from_numpy(inputs.values(n, bits)).cuda() if pairs else None
-M = args.M or (8192 if (pairs and bits == 64) else 16384)
+M = args.M or (8192 if (pairs and bits == 64) else (32768 if (bits == 32 and not pairs) else 16384))
 s = gss.Sorter(f"u{bits}", n, pairs, k=args.k, tile=args.tile, M=M, fill_div=args.fill_div or None)
 ko = torch.empty_like(k)
 vo = torch.empty_like(v) if pairs else None
