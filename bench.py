@@ -64,6 +64,14 @@ def auto_k(n: int, M: int) -> int:
     return k
 
 
+def auto_tile(n: int) -> int:
+    """The library's default tile (gss.h): 65536, halved while n < 296 tiles."""
+    T = 65536
+    while T > 2048 and n < T * 296:
+        T //= 2
+    return T
+
+
 def alg_bytes(kind: str, st, wk: int, wv: int, k: int, T: int, a: int, steps: int = 1) -> float:
     """Algorithmic bytes per step of one kernel kind."""
     split = sum(st.split_elems)
@@ -208,7 +216,7 @@ def run_ours(args, wl):
     wv = wk if pairs else 0
     kind = f"u{bits}"
     M = 8192 if (pairs and bits == 64) else (32768 if (bits == 32 and not pairs) else 16384)   # in-SM capacity (R5)
-    params = dict(k=auto_k(n, M), a=30, tile=65536, flags=16)   # flags 16: replay the launch sequence as a CUDA graph
+    params = dict(k=auto_k(n, M), a=30, tile=auto_tile(n), flags=16)   # flags 16: replay the launch sequence as a CUDA graph
     if wl == "c1_u32_2p16":
         params.update(k=128, k_policy="fixed")
     params["M"] = M

@@ -91,7 +91,8 @@ typedef struct gss_params {
   uint32_t oversample;      /* a; 0 -> 30                               */
   uint64_t small_threshold; /* M: buckets with m <= M go to the in-SM sort;       */
                             /* 0 -> the in-SM capacity of the type; at most that           */
-  uint32_t tile;            /* keys per tile T = t*l; multiple of 2048          */
+  uint32_t tile;            /* keys per tile T = t*l; multiple of 2048; 0 ->
+                               65536, halved while n < 296 tiles (min 2048)               */
   uint32_t max_levels;      /* distribution levels launched before the fallback; 0 -> auto */
   uint32_t k_policy;        /* 1 (default) adaptive k_b (R29), 2 = fixed k_b = k (paper)   */
   uint32_t fill_div;        /* adaptive rule divisor f (R29); 0 -> 4              */

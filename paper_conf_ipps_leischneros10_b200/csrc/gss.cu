@@ -32,7 +32,7 @@ gss_status gss_default_params(uint32_t key_bytes, uint32_t val_bytes, gss_params
   out->k = 0;                                   // n-dependent: 256, or 512 / 1024 for large n (see gss.h)
   out->oversample = 30;
   out->small_threshold = (val_bytes && key_bytes + val_bytes > 8) ? 8192 : 16384;
-  out->tile = 65536;
+  out->tile = 0;                                // n-dependent: 65536, smaller for small n (see gss.h)
   out->k_policy = 1;
   out->fill_div = 4;
   out->seed = 5489;

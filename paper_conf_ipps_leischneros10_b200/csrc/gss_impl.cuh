@@ -95,7 +95,14 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
     while (c->k < 1024 && (double)n > (double)c->k * c->k * (double)(c->M / 2)) c->k *= 2;
   }
   if (c->k < 2 || c->k > 1024 || (c->k & (c->k - 1))) return GSS_ERROR_INVALID_VALUE;
-  c->T = p.tile ? p.tile : 65536;
+  // default tile: 65536 keys, halved (down to 2048) while the input has fewer
+  // than 296 tiles (two CTAs per SM of a B200) so small sorts stay parallel
+  if (p.tile) {
+    c->T = p.tile;
+  } else {
+    c->T = 65536;
+    while (c->T > 2048 && n < (uint64_t)c->T * 296) c->T /= 2;
+  }
   if (c->T < 2048 || c->T % 2048 || c->T > (1u << 24)) return GSS_ERROR_INVALID_VALUE;
   c->k_policy = p.k_policy ? p.k_policy : 1;
   if (c->k_policy > 2) return GSS_ERROR_INVALID_VALUE;

@@ -63,7 +63,7 @@ def test_invalid_params_rejected(lib):
 def test_default_params(lib):
     p = gss._Params()
     assert lib.gss_default_params(8, 8, ctypes.byref(p)) == 0
-    assert (p.k, p.oversample, p.small_threshold, p.tile) == (0, 30, 8192, 65536)
+    assert (p.k, p.oversample, p.small_threshold, p.tile) == (0, 30, 8192, 0)
     assert lib.gss_default_params(4, 0, ctypes.byref(p)) == 0
     assert p.small_threshold == 16384
     assert lib.gss_default_params(3, 0, ctypes.byref(p)) == 1

@@ -17,7 +17,7 @@ ap.add_argument("--workload", default=bench.DEFAULT_WORKLOAD)
 ap.add_argument("--steps", type=int, default=1)
 ap.add_argument("--warmup", type=int, default=1)
 ap.add_argument("--k", type=int, default=0)                 # 0: the library default (auto)
-ap.add_argument("--tile", type=int, default=65536)
+ap.add_argument("--tile", type=int, default=0)                # 0: the library default
 ap.add_argument("--M", type=int, default=0)
 ap.add_argument("--fill_div", type=int, default=0)
 args = ap.parse_args()
