@@ -154,6 +154,31 @@ def mix_check(x: np.ndarray, y: np.ndarray) -> bool:
     return fp(x) == fp(y)
 
 
+def workload_params(wl: str):
+    """Sort parameters of a workload (the library defaults, stated explicitly so the
+    JSON line and the roofline terms can name them)."""
+    n, bits, pairs, _, _ = WORKLOADS[wl]
+    M = 8192 if (pairs and bits == 64) else (32768 if (bits == 32 and not pairs) else 16384)   # in-SM capacity (R5)
+    params = dict(k=auto_k(n, M), a=30, tile=auto_tile(n), flags=16)   # flags 16: replay the launch sequence as a CUDA graph
+    if wl == "c1_u32_2p16":
+        params.update(k=128, k_policy="fixed")
+    params["M"] = M
+    return params
+
+
+def metric_name(pairs: bool) -> str:
+    return f"sorting rate (Gkeys/s, {'key-value pairs' if pairs else 'keys'}); % HBM roofline"
+
+
+def config_dict(wl: str, world: int, params: dict) -> dict:
+    n, bits, pairs, distname, desc = WORKLOADS[wl]
+    kind = f"u{bits}"
+    return {"workload": wl, "description": desc, "n_per_gpu": n, "dist": distname, "key": kind,
+            "values": kind if pairs else None, **{k: v for k, v in params.items()},
+            "l2": "inputs larger than the 126 MB L2" if n * (bits // 8) > (256 << 20) else
+            "input fits in L2 (latency-bound config)", "parallelism": f"dp{world}"}
+
+
 # ---------------------------------------------------------------------------
 # reference arm: the CPU oracle
 # ---------------------------------------------------------------------------
@@ -167,9 +192,9 @@ def run_reference(args, wl):
     ns = min(n, REF_STEP_N)
     x = inputs.keys(dist, ns, bits, seed=1) if dist != "sorted" else inputs.keys(dist, ns, bits)
     v = inputs.values(ns, bits) if pairs else None
-    prm = oracle.Params(k=256, a=30, M=8192 if (pairs and bits == 64) else 16384, k_policy=1, fill_div=4, seed=5489)
-    if wl == "c1_u32_2p16":
-        prm.k, prm.k_policy = 128, 0
+    params = workload_params(wl)
+    prm = oracle.Params(k=params["k"], a=30, M=params["M"], k_policy=0 if params.get("k_policy") == "fixed" else 1,
+                        fill_div=4, seed=5489)
     times = []
     for i in range(args.warmup + args.steps):
         t0 = time.perf_counter()
@@ -180,11 +205,11 @@ def run_reference(args, wl):
     t = float(np.mean(times))
     val = ns / t / 1e9
     line = {
-        "impl": "reference", "metric": f"sorting rate (Gkeys/s, {'pairs' if pairs else 'keys'})", "value": val,
+        "impl": "reference", "metric": metric_name(pairs), "value": val,
         "unit": "Gkeys/s", "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
         "ms_per_step": t * 1e3, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
         "dtype": f"u{bits}", "data": "synthetic",
-        "config": {"workload": wl, "description": desc, "n_sample": ns, "dist": dist},
+        "config": {**config_dict(wl, 1, params), "n_sample": ns},
         "cpu_baseline": {"value": val, "unit": "Gkeys/s", "cores": 1, "kind": "oracle",
                          "sample": f"first {ns} keys of the workload's generator ({dist}, seed 1), one thread"},
         "e2e": {"value": val, "unit": "Gkeys/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
@@ -215,11 +240,8 @@ def run_ours(args, wl):
     wk = bits // 8
     wv = wk if pairs else 0
     kind = f"u{bits}"
-    M = 8192 if (pairs and bits == 64) else (32768 if (bits == 32 and not pairs) else 16384)   # in-SM capacity (R5)
-    params = dict(k=auto_k(n, M), a=30, tile=auto_tile(n), flags=16)   # flags 16: replay the launch sequence as a CUDA graph
-    if wl == "c1_u32_2p16":
-        params.update(k=128, k_policy="fixed")
-    params["M"] = M
+    params = workload_params(wl)
+    M = params["M"]
 
     # input: this rank's shard of the global input (weak scaling: n keys per GPU)
     x = inputs.keys(distname, n * world, bits, seed=1, start=rank * n, count=n)
@@ -355,14 +377,11 @@ def run_ours(args, wl):
 
     if rank == 0:
         line = {
-            "metric": f"sorting rate (Gkeys/s, {'key-value pairs' if pairs else 'keys'}); % HBM roofline",
+            "metric": metric_name(pairs),
             "value": round(value, 3), "unit": "Gkeys/s", "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": round(ms, 4), "higher_is_better": True, "scaling": "weak",
             "vs_baseline": None, "dtype": kind, "data": "synthetic",
-            "config": {"workload": wl, "description": desc, "n_per_gpu": n, "dist": distname, "key": kind,
-                       "values": kind if pairs else None, **{k: v for k, v in params.items()},
-                       "l2": "inputs larger than the 126 MB L2" if n * wk > (256 << 20) else
-                       "input fits in L2 (latency-bound config)", "parallelism": f"dp{world}"},
+            "config": config_dict(wl, world, params),
             "roofline": roof, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": gpu_launches,
             "clocks": clk.summary(), "result_check": bool(ok), **extra,
         }

@@ -24,6 +24,9 @@ constexpr int kClsThreads = 256;
 #ifndef GSS_SCATTER_EARLY
 #define GSS_SCATTER_EARLY 0
 #endif
+#ifndef GSS_SCATTER_PAIRFOLD
+#define GSS_SCATTER_PAIRFOLD 0   // 1: two threads per id in the fold (u64 3.18 vs 3.11 ms, pairs 3.30 vs 2.99: slower)
+#endif
 constexpr int kScatterThreads = GSS_SCATTER_THREADS;
 #ifndef GSS_SCATTER_ITER
 #define GSS_SCATTER_ITER 8
@@ -704,6 +707,32 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     GSS_PH(0);
     // chunk totals per id, exclusive scan over ids, then every warp's start
     // within each id folded into its counter (one lookup per key below)
+#if GSS_SCATTER_PAIRFOLD
+    if (2 * cur_K <= (uint32_t)kScatterThreads) {
+      // two threads per id, each folding half of the warps' counters (its
+      // 8 loads in flight at once); the pair's halves meet by a shuffle
+      constexpr int HW = NW / 2;
+      const uint32_t id = threadIdx.x >> 1, h = threadIdx.x & 1;
+      uint32_t x[HW], sh = 0;
+      if (id < cur_K) {
+#pragma unroll
+        for (int q = 0; q < HW; q++) { x[q] = wcnt[(h * HW + q) * kmax + id]; sh += x[q]; }
+      }
+      const uint32_t so = __shfl_xor_sync(kFull, sh, 1);
+      const uint32_t tot = sh + so;
+      const uint32_t ex0 = block_exclusive_scan<kScatterThreads>(h == 0 && id < cur_K ? tot : 0u, s_warp, nullptr);
+      const uint32_t ex = h == 0 ? ex0 : ex0 - tot;             // the id's run start (same for both halves)
+      if (id < cur_K) {
+        uint32_t run = ex + (h ? so : 0u);
+#pragma unroll
+        for (int q = 0; q < HW; q++) { wcnt[(h * HW + q) * kmax + id] = run; run += x[q]; }
+        if (h == 0) {
+          delta[id] = gbase[id] - ex;                           // global index = delta + staged position
+          gbase[id] += tot;
+        }
+      }
+    } else
+#endif
     {
       const uint32_t per = (cur_K + kScatterThreads - 1) / kScatterThreads;
       const uint32_t i0 = threadIdx.x * per;
