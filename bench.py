@@ -3,7 +3,8 @@
 the HBM roofline).
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--workload c4_u64_2p28|c2_u32_2p27|c3_u64_2p27|c3_kv64_2p27|c1_u32_2p16]
+                    [--workload c4_u64_2p28|c4_u64_2p29|c4_u64_2p30|c2_u32_2p27|c3_u64_2p27|c3_kv64_2p27|
+                                c1_u32_2p16|c5_kv64_2p29]
 
 One step = one full sort (every level of the k-way distribution pass plus the
 in-SM bucket sorts) of the workload's synthetic input, already resident in HBM
@@ -41,6 +42,8 @@ WORKLOADS = {
     "c3_u64_2p27": (1 << 27, 64, False, "uniform", "2^27 uniform u64 keys (BASELINE configs[2])"),
     "c3_kv64_2p27": (1 << 27, 64, True, "uniform", "2^27 uniform u64 key + u64 value pairs (BASELINE configs[2])"),
     "c1_u32_2p16": (1 << 16, 32, False, "uniform", "2^16 uniform u32 keys, k=128 (BASELINE configs[0]; launch-bound)"),
+    "c5_kv64_2p29": (1 << 29, 64, True, "uniform", "2^29 uniform u64 key + u64 value pairs per GPU: 2^32 on 8 GPUs "
+                     "(BASELINE configs[4]; distributed sample sort for N > 1)"),
 }
 DEFAULT_WORKLOAD = "c4_u64_2p28"
 CPU_SAMPLE_N = 1 << 26          # cpu_baseline leg: one oracle sort, ~10 s on one host core
