@@ -368,7 +368,13 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
   const int w = threadIdx.x >> 5;
   const uint32_t per = (nt + gridDim.x - 1) / gridDim.x;
   const uint32_t t0 = blockIdx.x * per, t1 = min(nt, t0 + per);
-  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + w * kmax);
+  // Counter arrays (the paper splits contention over 8 arrays).  Default: one per warp (8 per CTA,
+  // 32 threads each, as in the paper); -DGSS_CLS_NARR=1/2/4 shares arrays between warps (SURVEY NEXT-4 iii).
+#ifndef GSS_CLS_NARR
+#define GSS_CLS_NARR NW
+#endif
+  static_assert(NW % GSS_CLS_NARR == 0, "counter arrays must divide the warps");
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + (w / (NW / GSS_CLS_NARR)) * kmax);
   const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
   // node j of levels 5..7 is read by this lane at rep_b + 128 j
   const uint32_t rep_b = (uint32_t)__cvta_generic_to_shared(rep) - (1u << kTopLevels) * 128u +

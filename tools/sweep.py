@@ -10,9 +10,11 @@ import paper_conf_ipps_leischneros10_b200 as gss
 ap = argparse.ArgumentParser()
 ap.add_argument("--workload", default="c4_u64_2p28")
 ap.add_argument("--steps", type=int, default=5)
+ap.add_argument("--dist", default=None, help="override the workload's input distribution")
 ap.add_argument("cfgs", nargs="*")
 a = ap.parse_args()
 n, bits, pairs, dist, _ = bench.WORKLOADS[a.workload]
+dist = a.dist or dist
 x = inputs.keys(dist, n, bits, seed=1)
 k = torch.from_numpy(x).cuda()
 v = torch.from_numpy(inputs.values(n, bits)).cuda() if pairs else None
