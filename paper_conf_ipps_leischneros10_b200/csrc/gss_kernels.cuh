@@ -31,8 +31,15 @@ constexpr int kScatterThreads = GSS_SCATTER_THREADS;
 #ifndef GSS_SCATTER_ITER
 #define GSS_SCATTER_ITER 8
 #endif
-constexpr int kScatterIter = GSS_SCATTER_ITER;                      // keys per thread per chunk
-constexpr int kChunk = kScatterThreads * kScatterIter;            // 4096 keys staged per chunk
+#ifndef GSS_SCATTER_ITER_U32
+#define GSS_SCATTER_ITER_U32 16  // 4-byte keys alone: 16 per thread (the registers and shared bytes of 8 u64 keys);
+#endif                           // 2^27 u32 scatter 1.05 vs 1.14 ms (u64 at 16: 1.74 vs 1.56 ms, so 8 there)
+// keys per thread per chunk; a chunk (kScatterThreads x this) is staged in shared memory: 4096 keys, 8192 for u32
+template <class Key, class Val>
+constexpr int scatter_iter() { return (sizeof(Key) == 4 && !kHasVal<Val>) ? GSS_SCATTER_ITER_U32 : GSS_SCATTER_ITER; }
+#define GSS_SCATTER_CHUNK_CONSTANTS                                  \
+  constexpr int kScatterIter = scatter_iter<Key, Val>();            \
+  constexpr int kChunk = kScatterThreads * kScatterIter;
 constexpr int kScanCtas = 256;
 constexpr int kScanThreads = 256;
 constexpr int kPlanThreads = 256;
@@ -490,6 +497,7 @@ struct ScatterSmem {
     return (size_t)kmax * sizeof(Key) * 2 + (size_t)kRepNodes * 128;
   }
   static size_t bytes(uint32_t kmax, bool recompute = false) {
+    GSS_SCATTER_CHUNK_CONSTANTS
     size_t b = recompute ? tree_bytes(kmax) : 0;
     b += (size_t)kmax * 4 * 3;                                  // gbase, ctot, delta
     b += (size_t)(kScatterThreads / 32) * kmax * 4;             // per-warp counters
@@ -523,6 +531,10 @@ __device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t s
 template <class Key, class Val, class IdT, class Cmp, bool STABLE, bool RECOMP = false>
 __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
+  // the stable ranking (partitions, GSS_FLAG_STABLE) keeps 8 keys per thread: at 16 it spills (224 B stack);
+  // the shared allocation (ScatterSmem) is sized for the larger chunk
+  constexpr int kScatterIter = STABLE ? GSS_SCATTER_ITER : scatter_iter<Key, Val>();
+  constexpr int kChunk = kScatterThreads * kScatterIter;
   constexpr int NW = kScatterThreads / 32;
   constexpr uint32_t REP = rep_copies<Key>();
   Key* tree = reinterpret_cast<Key*>(smem_raw);
@@ -845,6 +857,7 @@ struct ScatterFastSmem {
 #endif
   static constexpr bool kStage = GSS_SCATTER_STAGE && (!kHasVal<Val> || sizeof(Key) + sizeof(Val) <= 8);
   static size_t bytes(uint32_t kmax) {
+    GSS_SCATTER_CHUNK_CONSTANTS
     size_t b = (size_t)kmax * 4 * 3;                            // cnt/off, delta, gbase
     b = (b + 15) & ~size_t(15);
     b += (size_t)kChunk * sizeof(Key) * (kStage ? 2 : 1);
@@ -858,6 +871,7 @@ template <class Key, class Val, class IdT, class Cmp>
 __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     k_scatter_fast(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
+  GSS_SCATTER_CHUNK_CONSTANTS
   constexpr bool STAGE = ScatterFastSmem<Key, Val, IdT>::kStage;
   uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw);          // chunk counts, then run offsets
   uint32_t* delta = cnt + kmax;
