@@ -3,7 +3,7 @@
 the HBM roofline).
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--workload c4_u64_2p28|c4_u64_2p29|c4_u64_2p30|c2_u32_2p27|c3_u64_2p27|c3_kv64_2p27|
+                    [--workload c4_u64_2p28|c4_u64_2p29|c4_u64_2p30|c2_u32_2p27|c3_u64_2p27|c3_kv64_2p27|c3_kv32_2p27|
                                 c1_u32_2p16|c5_kv64_2p29]
 
 One step = one full sort (every level of the k-way distribution pass plus the
@@ -41,6 +41,7 @@ WORKLOADS = {
     "c2_u32_2p27": (1 << 27, 32, False, "uniform", "2^27 uniform u32 keys (BASELINE configs[1])"),
     "c3_u64_2p27": (1 << 27, 64, False, "uniform", "2^27 uniform u64 keys (BASELINE configs[2])"),
     "c3_kv64_2p27": (1 << 27, 64, True, "uniform", "2^27 uniform u64 key + u64 value pairs (BASELINE configs[2])"),
+    "c3_kv32_2p27": (1 << 27, 32, True, "uniform", "2^27 uniform u32 key + u32 value pairs (not a BASELINE config)"),
     "c1_u32_2p16": (1 << 16, 32, False, "uniform", "2^16 uniform u32 keys, k=128 (BASELINE configs[0]; launch-bound)"),
     "c5_kv64_2p29": (1 << 29, 64, True, "uniform", "2^29 uniform u64 key + u64 value pairs per GPU: 2^32 on 8 GPUs "
                      "(BASELINE configs[4]; distributed sample sort for N > 1)"),

@@ -35,8 +35,15 @@ constexpr int kScatterThreads = GSS_SCATTER_THREADS;
 #define GSS_SCATTER_ITER_U32 16  // 4-byte keys alone: 16 per thread (the registers and shared bytes of 8 u64 keys);
 #endif                           // 2^27 u32 scatter 1.05 vs 1.14 ms (u64 at 16: 1.74 vs 1.56 ms, so 8 there)
 // keys per thread per chunk; a chunk (kScatterThreads x this) is staged in shared memory: 4096 keys, 8192 for u32
+#ifndef GSS_SCATTER_ITER_KV32
+#define GSS_SCATTER_ITER_KV32 8
+#endif
 template <class Key, class Val>
-constexpr int scatter_iter() { return (sizeof(Key) == 4 && !kHasVal<Val>) ? GSS_SCATTER_ITER_U32 : GSS_SCATTER_ITER; }
+constexpr int scatter_iter() {
+  return sizeof(Key) == 4 ? (kHasVal<Val> ? (sizeof(Val) == 4 ? GSS_SCATTER_ITER_KV32 : GSS_SCATTER_ITER)
+                                          : GSS_SCATTER_ITER_U32)
+                          : GSS_SCATTER_ITER;
+}
 #define GSS_SCATTER_CHUNK_CONSTANTS                                  \
   constexpr int kScatterIter = scatter_iter<Key, Val>();            \
   constexpr int kChunk = kScatterThreads * kScatterIter;
