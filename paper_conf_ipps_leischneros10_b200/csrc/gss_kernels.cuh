@@ -15,6 +15,9 @@
 namespace gss {
 
 constexpr int kClsThreads = 256;
+#ifndef GSS_CLS_U
+#define GSS_CLS_U 8                                              // keys per lane per classify group
+#endif
 #ifndef GSS_SCATTER_THREADS
 #define GSS_SCATTER_THREADS 512
 #endif
@@ -211,7 +214,7 @@ constexpr uint32_t rep_copies() { return 128u / sizeof(Key); }
 template <class Key>
 constexpr size_t cls_smem_bytes(uint32_t kmax) {
   return (size_t)kmax * sizeof(Key) * 2 + (size_t)kRepNodes * 128 + (size_t)(kClsThreads / 32) * kmax * 4 +
-         (size_t)(kClsThreads / 32) * 256 * 2;
+         (size_t)(kClsThreads / 32) * (32 * GSS_CLS_U) * 2;
 }
 
 // One level of Algorithm 2 (j := 2j + (e > bt[j])) on a node address
@@ -293,9 +296,6 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
                                               uint32_t len, uint32_t tree_s, uint32_t rep_b, const Key* spl,
                                               uint32_t logk, uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid,
                                               Cmp less) {
-#ifndef GSS_CLS_U
-#define GSS_CLS_U 8
-#endif
   constexpr int U = GSS_CLS_U;                                 // keys per lane per group
   constexpr uint32_t G = U * kClsThreads;                      // keys per group
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
@@ -330,8 +330,11 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
       *reinterpret_cast<uint32_t*>(gp) = *reinterpret_cast<const uint32_t*>(wid + lane * U);
     } else if constexpr (U * sizeof(IdT) == 8) {
       *reinterpret_cast<uint2*>(gp) = *reinterpret_cast<const uint2*>(wid + lane * U);
+    } else if constexpr (U * sizeof(IdT) == 32) {
+      *reinterpret_cast<uint4*>(gp) = *reinterpret_cast<const uint4*>(wid + lane * U);
+      *reinterpret_cast<uint4*>(gp + 16 / sizeof(IdT)) = *reinterpret_cast<const uint4*>(wid + lane * U + 16 / sizeof(IdT));
     } else {
-      static_assert(U * sizeof(IdT) == 16, "ids per lane: 4, 8 or 16 bytes");
+      static_assert(U * sizeof(IdT) == 16, "ids per lane: 4, 8, 16 or 32 bytes");
       *reinterpret_cast<uint4*>(gp) = *reinterpret_cast<const uint4*>(wid + lane * U);
     }
     __syncwarp();
@@ -374,7 +377,7 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
   Key* rep = spl + kmax;                                       // kRepNodes x REP keys
   uint32_t* wcnt = reinterpret_cast<uint32_t*>(rep + kRepNodes * REP);
   constexpr int NW = kClsThreads / 32;
-  IdT* wid = reinterpret_cast<IdT*>(wcnt + NW * kmax) + (threadIdx.x >> 5) * 256;   // per-warp id staging
+  IdT* wid = reinterpret_cast<IdT*>(wcnt + NW * kmax) + (threadIdx.x >> 5) * (32 * GSS_CLS_U);   // per-warp id staging
   const Cmp less;
   const uint32_t slot = level & 1;
   const uint32_t nt = c.cnt->lvl[level].num_tiles;
