@@ -21,13 +21,23 @@ import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "oracle.c")
+_REF = os.path.join(_HERE, "libref.cc")
 _LIB = os.path.join(_HERE, "liboracle.so")
 
 
 def build(force: bool = False) -> str:
-    """Compile oracle.c with gcc (plain -O2, no vectorisation tricks)."""
-    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
-        subprocess.check_call(["gcc", "-O2", "-Wall", "-shared", "-fPIC", "-o", _LIB, _SRC])
+    """Compile oracle.c with gcc (plain -O2, no vectorisation tricks; OpenMP only
+    for the thread-parallel timing mode) plus the library-sort references."""
+    newest = max(os.path.getmtime(_SRC), os.path.getmtime(_REF), os.path.getmtime(__file__))
+    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < newest:
+        tmp = _LIB + f".{os.getpid()}.tmp"
+        o1, o2 = tmp + ".oracle.o", tmp + ".libref.o"
+        subprocess.check_call(["gcc", "-O2", "-Wall", "-fopenmp", "-fPIC", "-c", "-o", o1, _SRC])
+        subprocess.check_call(["g++", "-O2", "-Wall", "-fopenmp", "-fPIC", "-c", "-o", o2, _REF])
+        subprocess.check_call(["g++", "-shared", "-fopenmp", "-o", tmp, o1, o2])
+        os.replace(tmp, _LIB)
+        for o in (o1, o2):
+            os.remove(o)
     return _LIB
 
 
@@ -39,7 +49,7 @@ class _Params(ctypes.Structure):
         ("k_policy", ctypes.c_uint32),
         ("fill_div", ctypes.c_uint32),
         ("sample_cap", ctypes.c_uint32),
-        ("pad0", ctypes.c_uint32),
+        ("threads", ctypes.c_uint32),
         ("seed", ctypes.c_uint64),
     ]
 
@@ -85,6 +95,11 @@ def _load():
         lib.oracle_log_free.argtypes = [vp]
         lib.oracle_select.restype = u64
         lib.oracle_select.argtypes = [vp, u64, u64]
+        for w in ("u32", "u64"):
+            getattr(lib, f"libref_std_sort_{w}").restype = None
+            getattr(lib, f"libref_std_sort_{w}").argtypes = [vp, u64]
+            getattr(lib, f"libref_parallel_sort_{w}").restype = None
+            getattr(lib, f"libref_parallel_sort_{w}").argtypes = [vp, u64, ctypes.c_int]
         _lib = lib
     return _lib
 
@@ -100,9 +115,10 @@ class Params:
     fill_div: int = 4
     sample_cap: int = 16384
     seed: int = 5489        # R2
+    threads: int = 1        # > 1: OpenMP tasks over child buckets (same output, for timing)
 
     def c(self) -> _Params:
-        return _Params(self.k, self.a, self.M, self.k_policy, self.fill_div, self.sample_cap, 0,
+        return _Params(self.k, self.a, self.M, self.k_policy, self.fill_div, self.sample_cap, self.threads,
                        self.seed & 0xFFFFFFFFFFFFFFFF)
 
 
@@ -227,3 +243,16 @@ def select(keys, r: int) -> int:
     """The rank-r element of keys (the r-th entry of the sorted output)."""
     k = _as_u64(keys)
     return int(_load().oracle_select(_ptr(k), k.size, r))
+
+
+def library_sort(keys: np.ndarray, threads: int = 1) -> np.ndarray:
+    """CPU library reference (not the oracle): std::sort (threads == 1) or
+    __gnu_parallel::sort on `threads` threads, on a copy of keys."""
+    a = np.ascontiguousarray(np.array(keys, copy=True))
+    w = {np.dtype(np.uint32): "u32", np.dtype(np.uint64): "u64"}[a.dtype]
+    lib = _load()
+    if threads <= 1:
+        getattr(lib, f"libref_std_sort_{w}")(_ptr(a), a.size)
+    else:
+        getattr(lib, f"libref_parallel_sort_{w}")(_ptr(a), a.size, threads)
+    return a

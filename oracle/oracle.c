@@ -15,6 +15,14 @@
  * zero-extends, which preserves order and equality); values, when present,
  * are uint64_t payloads that travel with their keys.
  *
+ * Threads (timing only): with params.threads > 1 the
+ * child buckets of a level are sorted as independent OpenMP tasks, and a
+ * large bucket's Phases 2-4 run over chunks (per-chunk counts, the
+ * bucket-major exclusive scan over (bucket, chunk), then a stable
+ * per-chunk placement -- the CPU analogue of P:256-263).  Each step is the
+ * same plain computation; the output and the level records (sorted by
+ * (level, lo)) are identical for any thread count (test_oracle.py).
+ *
  * Parity pins (tests/test_oracle.py): brute force / library sort on every
  * input of length <= 6 over {0,1,2}; the paper's k=8 tree layout (P:295-304,
  * tests/golden/tree_k8.txt); Algorithm 2 == lower_bound; SplitMix64 known
@@ -24,6 +32,7 @@
 #include <stdint.h>
 #include <stdlib.h>
 #include <string.h>
+#include <omp.h>
 
 /* ------------------------------------------------------------------ */
 /* Parameters (paper defaults)          */
@@ -35,7 +44,7 @@ typedef struct oracle_params {
   uint32_t k_policy;   /* 0 = fixed k_b = k (the paper); 1 = adaptive (R29)             */
   uint32_t fill_div;   /* adaptive rule: k_b = min(k, max(4, pow2ceil(ceil(f*m/M))))    */
   uint32_t sample_cap; /* a_eff = min(a, sample_cap / k_b), at least 1 (smem bound, R9) */
-  uint32_t pad0;
+  uint32_t threads;    /* 0/1 sequential; > 1: OpenMP tasks over child buckets (timing)  */
   uint64_t seed;       /* sampling seed (R2)                                             */
 } oracle_params;
 
@@ -182,11 +191,23 @@ static void small_sort(uint64_t* A, uint64_t* V, uint64_t m) {
 /* ------------------------------------------------------------------ */
 static void log_push(oracle_log* lg, const oracle_record* r) {
   if (!lg) return;
-  if (lg->n == lg->cap) {
-    lg->cap = lg->cap ? 2 * lg->cap : 64;
-    lg->r = (oracle_record*)realloc(lg->r, lg->cap * sizeof(oracle_record));
+#pragma omp critical(oracle_log)
+  {
+    if (lg->n == lg->cap) {
+      lg->cap = lg->cap ? 2 * lg->cap : 64;
+      lg->r = (oracle_record*)realloc(lg->r, lg->cap * sizeof(oracle_record));
+    }
+    lg->r[lg->n++] = *r;
   }
-  lg->r[lg->n++] = *r;
+}
+
+/* Records in (level, lo) order: the sequential recursion's order does not
+ * survive tasks, this one is the same for any thread count. */
+static int cmp_rec(const void* a, const void* b) {
+  const oracle_record* x = (const oracle_record*)a;
+  const oracle_record* y = (const oracle_record*)b;
+  if (x->level != y->level) return (x->level > y->level) - (x->level < y->level);
+  return (x->lo > y->lo) - (x->lo < y->lo);
 }
 
 /* ------------------------------------------------------------------ */
@@ -198,8 +219,54 @@ typedef struct step_out {
   uint64_t* child;    /* K    */
 } step_out;
 
+/* Phases 2-4 of one bucket over fixed chunks of PAR_CHUNK elements (used
+ * with threads > 1 only): ids and per-chunk counts, then the exclusive scan
+ * in bucket-major order over (bucket, chunk) -- the paper's k x p table
+ * (R6) -- then every chunk places its elements in input order.
+ * The result is the same stable partition as the sequential loops. */
+#define PAR_CHUNK ((uint64_t)1 << 16)
+#define PAR_MIN_ELEMS ((uint64_t)1 << 18)
+static void distribute_chunks(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, const uint64_t* spl,
+                              uint32_t ks, uint32_t eq, uint32_t K, uint64_t** cnt_out) {
+  const uint64_t nch = (m + PAR_CHUNK - 1) / PAR_CHUNK;
+  uint32_t* id = (uint32_t*)malloc(m * sizeof(uint32_t));
+  uint64_t* h = (uint64_t*)calloc(nch * K, sizeof(uint64_t));      /* h[c*K + b] */
+#pragma omp taskloop grainsize(1)
+  for (uint64_t c = 0; c < nch; c++) {
+    const uint64_t e = (c + 1) * PAR_CHUNK < m ? (c + 1) * PAR_CHUNK : m;
+    for (uint64_t i = c * PAR_CHUNK; i < e; i++) {
+      id[i] = oracle_classify(spl, ks - 1, eq, A[lo + i]);
+      h[c * K + id[i]]++;
+    }
+  }
+  uint64_t* cnt = (uint64_t*)calloc(K, sizeof(uint64_t));
+  uint64_t run = 0;
+  for (uint32_t b = 0; b < K; b++)
+    for (uint64_t c = 0; c < nch; c++) {
+      const uint64_t x = h[c * K + b];
+      h[c * K + b] = run;
+      run += x;
+      cnt[b] += x;
+    }
+  uint64_t* TA = (uint64_t*)malloc(m * sizeof(uint64_t));
+  uint64_t* TV = V ? (uint64_t*)malloc(m * sizeof(uint64_t)) : NULL;
+#pragma omp taskloop grainsize(1)
+  for (uint64_t c = 0; c < nch; c++) {
+    const uint64_t e = (c + 1) * PAR_CHUNK < m ? (c + 1) * PAR_CHUNK : m;
+    for (uint64_t i = c * PAR_CHUNK; i < e; i++) {
+      uint64_t d = h[c * K + id[i]]++;
+      TA[d] = A[lo + i];
+      if (V) TV[d] = V[lo + i];
+    }
+  }
+  memcpy(A + lo, TA, m * sizeof(uint64_t));
+  if (V) memcpy(V + lo, TV, m * sizeof(uint64_t));
+  free(TA); free(TV); free(h); free(id);
+  *cnt_out = cnt;
+}
+
 static void distribute(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, uint32_t level,
-                       const oracle_params* p, step_out* o) {
+                       const oracle_params* p, step_out* o, int par) {
   /* Phase 1: random sample S of a*k elements (R1, R2), sorted. */
   uint32_t kb = oracle_choose_kb(p, m);
   uint32_t a = oracle_a_eff(p, kb);
@@ -223,30 +290,35 @@ static void distribute(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, uint32
   }
   uint32_t K = eq ? 2 * ks - 1 : ks;
   free(S);
+  uint64_t* cnt;
 
-  /* Phase 2: bucket index of every element and the bucket sizes. */
-  uint32_t* id = (uint32_t*)malloc(m * sizeof(uint32_t));
-  uint64_t* cnt = (uint64_t*)calloc(K, sizeof(uint64_t));
-  for (uint64_t i = 0; i < m; i++) {
-    id[i] = oracle_classify(spl, ks - 1, eq, A[lo + i]);
-    cnt[id[i]]++;
+  if (par && m >= PAR_MIN_ELEMS) {
+    distribute_chunks(A, V, lo, m, spl, ks, eq, K, &cnt);
+  } else {
+    /* Phase 2: bucket index of every element and the bucket sizes. */
+    uint32_t* id = (uint32_t*)malloc(m * sizeof(uint32_t));
+    cnt = (uint64_t*)calloc(K, sizeof(uint64_t));
+    for (uint64_t i = 0; i < m; i++) {
+      id[i] = oracle_classify(spl, ks - 1, eq, A[lo + i]);
+      cnt[id[i]]++;
+    }
+    /* Phase 3: exclusive prefix sum over the bucket sizes. */
+    uint64_t* off = (uint64_t*)malloc(K * sizeof(uint64_t));
+    uint64_t run = 0;
+    for (uint32_t b = 0; b < K; b++) { off[b] = run; run += cnt[b]; }
+    /* Phase 4: place every element at its bucket's next free slot, in input
+     * order -- a stable partition (R7). */
+    uint64_t* TA = (uint64_t*)malloc(m * sizeof(uint64_t));
+    uint64_t* TV = V ? (uint64_t*)malloc(m * sizeof(uint64_t)) : NULL;
+    for (uint64_t i = 0; i < m; i++) {
+      uint64_t d = off[id[i]]++;
+      TA[d] = A[lo + i];
+      if (V) TV[d] = V[lo + i];
+    }
+    memcpy(A + lo, TA, m * sizeof(uint64_t));
+    if (V) memcpy(V + lo, TV, m * sizeof(uint64_t));
+    free(TA); free(TV); free(off); free(id);
   }
-  /* Phase 3: exclusive prefix sum over the bucket sizes. */
-  uint64_t* off = (uint64_t*)malloc(K * sizeof(uint64_t));
-  uint64_t run = 0;
-  for (uint32_t b = 0; b < K; b++) { off[b] = run; run += cnt[b]; }
-  /* Phase 4: place every element at its bucket's next free slot, in input
-   * order -- a stable partition (R7). */
-  uint64_t* TA = (uint64_t*)malloc(m * sizeof(uint64_t));
-  uint64_t* TV = V ? (uint64_t*)malloc(m * sizeof(uint64_t)) : NULL;
-  for (uint64_t i = 0; i < m; i++) {
-    uint64_t d = off[id[i]]++;
-    TA[d] = A[lo + i];
-    if (V) TV[d] = V[lo + i];
-  }
-  memcpy(A + lo, TA, m * sizeof(uint64_t));
-  if (V) memcpy(V + lo, TV, m * sizeof(uint64_t));
-  free(TA); free(TV); free(off); free(id);
 
   o->kb = kb; o->ks = ks; o->eq = eq; o->K = K; o->a_eff = a;
   o->spl = spl; o->child = cnt;
@@ -255,14 +327,15 @@ static void distribute(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, uint32
 /* ------------------------------------------------------------------ */
 /* Algorithm 1 SampleSort, with delayed small sorts */
 /* ------------------------------------------------------------------ */
+#define TASK_MIN_ELEMS 4096
 static void sort_range(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, uint32_t level,
-                       const oracle_params* p, oracle_log* lg) {
+                       const oracle_params* p, oracle_log* lg, int par) {
   if (m <= p->M) {                              /* "if n < M then SmallSort" (R5) */
     small_sort(A + lo, V ? V + lo : NULL, m);
     return;
   }
   step_out o;
-  distribute(A, V, lo, m, level, p, &o);
+  distribute(A, V, lo, m, level, p, &o, par);
   oracle_record r;
   r.level = level; r.kb = o.kb; r.ks = o.ks; r.eq = o.eq; r.K = o.K; r.a_eff = o.a_eff;
   r.lo = lo; r.m = m; r.spl = o.spl; r.child = o.child;
@@ -271,9 +344,18 @@ static void sort_range(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, uint32
   uint64_t c = lo;
   for (uint32_t b = 0; b < o.K; b++) {
     uint64_t cm = o.child[b];
-    if (!(o.eq && (b & 1)))                     /* equality buckets hold one key value: final (R4) */
-      sort_range(A, V, c, cm, level + 1, p, lg);
+    if (!(o.eq && (b & 1))) {                   /* equality buckets hold one key value: final (R4) */
+      if (par && cm >= TASK_MIN_ELEMS) {
+#pragma omp task firstprivate(c, cm)
+        sort_range(A, V, c, cm, level + 1, p, lg, par);
+      } else {
+        sort_range(A, V, c, cm, level + 1, p, lg, par);
+      }
+    }
     c += cm;
+  }
+  if (par) {
+#pragma omp taskwait
   }
   if (!lg) { free(o.spl); free(o.child); }
 }
@@ -287,7 +369,14 @@ static void sort_range(uint64_t* A, uint64_t* V, uint64_t lo, uint64_t m, uint32
  * step (free with oracle_log_free); otherwise returns NULL. */
 void* oracle_sort(uint64_t* keys, uint64_t* vals, uint64_t n, const oracle_params* p, int want_log) {
   oracle_log* lg = want_log ? (oracle_log*)calloc(1, sizeof(oracle_log)) : NULL;
-  sort_range(keys, vals, 0, n, 0, p, lg);
+  if (p->threads > 1) {
+#pragma omp parallel num_threads(p->threads)
+#pragma omp single
+    sort_range(keys, vals, 0, n, 0, p, lg, 1);
+  } else {
+    sort_range(keys, vals, 0, n, 0, p, lg, 0);
+  }
+  if (lg && lg->n > 1) qsort(lg->r, lg->n, sizeof(oracle_record), cmp_rec);
   return lg;
 }
 
@@ -297,7 +386,7 @@ void* oracle_sort(uint64_t* keys, uint64_t* vals, uint64_t n, const oracle_param
 void* oracle_distribute(uint64_t* keys, uint64_t* vals, uint64_t n, const oracle_params* p) {
   oracle_log* lg = (oracle_log*)calloc(1, sizeof(oracle_log));
   step_out o;
-  distribute(keys, vals, 0, n, 0, p, &o);
+  distribute(keys, vals, 0, n, 0, p, &o, 0);
   oracle_record r;
   r.level = 0; r.kb = o.kb; r.ks = o.ks; r.eq = o.eq; r.K = o.K; r.a_eff = o.a_eff;
   r.lo = 0; r.m = n; r.spl = o.spl; r.child = o.child;

@@ -262,3 +262,79 @@ def test_select_is_rank(oracle_mod):
     s = np.sort(x)
     for r in (0, 1, 777, 10_000, 20_000):
         assert oracle_mod.select(x, r) == int(s[r])
+
+
+# --------------------------------------------------------------------------
+# Equality mode (R4) splitters, recomputed from the hashed sample in Python,
+# at level 0 and at level 1 (lo != 0 keys the hash); R4.
+# --------------------------------------------------------------------------
+def py_splitters(arr, lo, m, level, p, kb, a):
+    """Sample a*kb keys of arr[lo, lo+m) at H(seed, level, lo, j) (R2), sort
+    them, take S[a(i+1)-1] (R1); if two are equal or kb == 2, switch to
+    equality mode with ks = max(2, kb/2) splitters S[(s/ks)(i+1)-1] (R4)."""
+    h0 = py_fmix((py_fmix((p.seed ^ (level << 56)) + GAMMA) ^ lo) + GAMMA)
+    s = a * kb
+    S = sorted(int(arr[lo + ((py_fmix((h0 ^ j) + GAMMA) * m) >> 64)]) for j in range(s))
+    spl = [S[a * (i + 1) - 1] for i in range(kb - 1)]
+    eq = kb == 2 or any(spl[i] == spl[i + 1] for i in range(len(spl) - 1))
+    if not eq:
+        return 0, kb, spl
+    ks = max(2, kb // 2)
+    stride = s // ks
+    return 1, ks, [S[stride * (i + 1) - 1] for i in range(ks - 1)]
+
+
+@pytest.mark.parametrize("dist", ["dd", "and5", "equal", "uniform"])
+def test_equality_mode_splitters_recomputed(oracle_mod, dist):
+    n = 40_000
+    x = inputs.keys(dist, n, 32, seed=12)
+    if dist == "uniform":
+        x = (x % np.uint32(7)).astype(np.uint32)                  # few distinct keys: eq mode at level 0
+    p = oracle_mod.Params(k=64, a=12, M=256, k_policy=0, seed=321)
+    lvl1, _, r0 = oracle_mod.distribute(x, None, p)
+    eq, ks, spl = py_splitters(x, 0, n, 0, p, r0.kb, r0.a_eff)
+    assert (r0.eq, r0.ks) == (eq, ks)
+    assert [int(s) for s in r0.splitters] == spl
+    saw_eq = r0.eq
+    # level-1 buckets: the oracle's own records of the whole sort, against the
+    # Python recomputation on the (separately pinned) level-0 partition
+    _, _, recs = oracle_mod.sort(x, params=p, log=True)
+    assert recs[0].lo == 0 and recs[0].level == 0
+    for r in recs:
+        if r.level != 1:
+            continue
+        eq, ks, spl = py_splitters(lvl1, r.lo, r.m, 1, p, r.kb, r.a_eff)
+        assert (r.eq, r.ks, r.K) == (eq, ks, 2 * ks - 1 if eq else ks)
+        assert [int(s) for s in r.splitters] == spl
+        saw_eq |= r.eq
+    assert saw_eq, "input did not exercise equality mode"
+
+
+@pytest.mark.parametrize("pairs", [False, True])
+def test_threads_give_identical_results(oracle_mod, pairs):
+    """The OpenMP mode (tasks per child bucket, chunked Phases 2-4) gives the
+    same keys, values and level records as the sequential recursion."""
+    n = 600_001
+    for dist in ("uniform", "dd", "and3"):
+        x = inputs.keys(dist, n, 64, seed=3)
+        v = inputs.values(n, 64) if pairs else None
+        res = []
+        for t in (1, 4):
+            p = oracle_mod.Params(k=64, a=20, M=2000, k_policy=1, seed=7, threads=t)
+            res.append(oracle_mod.sort(x, v, p, log=True))
+        (k1, v1, r1), (k4, v4, r4) = res
+        np.testing.assert_array_equal(k1, np.sort(x))
+        np.testing.assert_array_equal(k1, k4)
+        if pairs:
+            np.testing.assert_array_equal(v1, v4)
+        assert len(r1) == len(r4) and len(r1) > 1
+        for a, b in zip(r1, r4):
+            assert (a.level, a.lo, a.m, a.kb, a.ks, a.eq, a.K) == (b.level, b.lo, b.m, b.kb, b.ks, b.eq, b.K)
+            np.testing.assert_array_equal(a.splitters, b.splitters)
+            np.testing.assert_array_equal(a.children, b.children)
+
+
+def test_library_references_sort(oracle_mod):
+    x = inputs.keys("uniform", 100_003, 32, seed=2)
+    for t in (1, 3):
+        np.testing.assert_array_equal(oracle_mod.library_sort(x, t), np.sort(x))
