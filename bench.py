@@ -47,8 +47,8 @@ WORKLOADS = {
                      "(BASELINE configs[4]; distributed sample sort for N > 1)"),
 }
 DEFAULT_WORKLOAD = "c4_u64_2p28"
-CPU_SAMPLE_N = 1 << 26          # cpu_baseline leg: one oracle sort, ~10 s on one host core
-REF_STEP_N = 1 << 24            # --impl reference: per-step sample, ~2.5 s per step
+CPU_SAMPLE_N = 1 << 25          # cpu_baseline leg: one oracle sort per thread count (~5 s on one core)
+REF_STEP_N = 1 << 25            # --impl reference: per-step sample on all host cores
 
 
 def peaks():
@@ -158,6 +158,57 @@ def mix_check(x: np.ndarray, y: np.ndarray) -> bool:
     return fp(x) == fp(y)
 
 
+def pairs_check(x: np.ndarray, ko: np.ndarray, vo: np.ndarray, v0: int = 0) -> bool:
+    """Values are input indices (+ v0, R20): they must form a permutation and
+    carry their own key: x[v - v0] == key (result check, not timed)."""
+    idx = vo.astype(np.int64) - v0
+    if idx.min(initial=0) < 0 or idx.max(initial=0) >= x.size:
+        return False
+    seen = np.zeros(x.size, dtype=bool)
+    seen[idx] = True
+    return bool(seen.all()) and bool(np.array_equal(x[idx], ko))
+
+
+def cpu_model() -> str:
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
+def cpu_baseline(wl: str, x: np.ndarray, hv, params: dict) -> dict:
+    """The oracle on this host's cores, on a bounded sample of the workload
+    (SURVEY 8(d) d.8): all cores (OpenMP tasks per child bucket, the line's
+    value), one thread, and the library sorts std::sort (1 thread) and
+    __gnu_parallel::sort (all cores) as context.  Not tuned; a baseline only."""
+    import oracle
+    oracle.build()
+    n, bits, pairs, distname, _ = WORKLOADS[wl]
+    ns = min(n, CPU_SAMPLE_N)
+    xs = x[:ns] if distname != "sorted" else inputs.keys(distname, ns, bits)
+    vs = hv[:ns] if pairs else None
+    cores = os.cpu_count() or 1
+    out = {}
+    for label, thr in (("all_cores", cores), ("one_thread", 1)):
+        prm = oracle.Params(k=params["k"], a=30, M=params["M"], k_policy=0 if params.get("k_policy") == "fixed" else 1,
+                            fill_div=4, seed=5489, threads=thr)
+        t0 = time.perf_counter()
+        oracle.sort(xs, vs, prm)
+        out[label] = {"value": ns / (time.perf_counter() - t0) / 1e9, "threads": thr}
+    lib = {}
+    if not pairs:
+        for label, thr in (("std_sort", 1), ("gnu_parallel_sort", cores)):
+            t0 = time.perf_counter()
+            oracle.library_sort(xs, thr)
+            lib[label] = {"value": ns / (time.perf_counter() - t0) / 1e9, "threads": thr}
+    return {"value": out["all_cores"]["value"], "unit": "Gkeys/s", "cores": cores, "kind": "oracle",
+            "sample": f"first {ns} keys of this workload's input ({distname}, seed 1); one oracle sort per thread count",
+            "one_thread": out["one_thread"], "library_refs": lib, "cpu_model": cpu_model()}
+
+
 def workload_params(wl: str):
     """Sort parameters of a workload (the library defaults, stated explicitly so the
     JSON line and the roofline terms can name them)."""
@@ -197,8 +248,9 @@ def run_reference(args, wl):
     x = inputs.keys(dist, ns, bits, seed=1) if dist != "sorted" else inputs.keys(dist, ns, bits)
     v = inputs.values(ns, bits) if pairs else None
     params = workload_params(wl)
+    cores = os.cpu_count() or 1
     prm = oracle.Params(k=params["k"], a=30, M=params["M"], k_policy=0 if params.get("k_policy") == "fixed" else 1,
-                        fill_div=4, seed=5489)
+                        fill_div=4, seed=5489, threads=cores)
     times = []
     for i in range(args.warmup + args.steps):
         t0 = time.perf_counter()
@@ -214,8 +266,9 @@ def run_reference(args, wl):
         "ms_per_step": t * 1e3, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
         "dtype": f"u{bits}", "data": "synthetic",
         "config": {**config_dict(wl, 1, params), "n_sample": ns},
-        "cpu_baseline": {"value": val, "unit": "Gkeys/s", "cores": 1, "kind": "oracle",
-                         "sample": f"first {ns} keys of the workload's generator ({dist}, seed 1), one thread"},
+        "cpu_baseline": {"value": val, "unit": "Gkeys/s", "cores": cores, "kind": "oracle",
+                         "sample": f"first {ns} keys of the workload's generator ({dist}, seed 1), "
+                                   f"{cores} threads (OpenMP tasks per child bucket)", "cpu_model": cpu_model()},
         "e2e": {"value": val, "unit": "Gkeys/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -297,6 +350,8 @@ def run_ours(args, wl):
     # ---- result check (not timed) ----
     if not use_dist:
         ok = mix_check(x, kout.cpu().numpy())
+        if pairs:
+            ok = ok and pairs_check(x, kout.cpu().numpy(), vout.cpu().numpy(), rank * n)
     else:
         ok = sorter.verify(x)
 
@@ -359,6 +414,8 @@ def run_ours(args, wl):
         torch.cuda.synchronize(dev)
         ems = e0.elapsed_time(e1) / ke
         ok = ok and bool(np.array_equal(ho.numpy(), kout.cpu().numpy()))
+        if pairs:
+            ok = ok and pairs_check(x, ho.numpy(), hvo.numpy(), rank * n)
         e2e = {"value": n / (ems * 1e-3) / 1e9, "unit": "Gkeys/s", "h2d_bytes_per_step": n * (wk + wv),
                "d2h_bytes_per_step": n * (wk + wv), "ms_per_step": ems,
                "path": "gss_host_pipeline_run: pinned host in/out, H2D + sort + D2H every step, steps pipelined"}
@@ -366,18 +423,7 @@ def run_ours(args, wl):
     # ---- CPU baseline: the oracle on a bounded sample (rank 0, N == 1 only) ----
     cpu = None
     if world == 1 and not use_dist and not args.no_cpu_baseline:
-        import oracle
-        oracle.build()
-        ns = min(n, CPU_SAMPLE_N)
-        xs = x[:ns] if distname != "sorted" else inputs.keys(distname, ns, bits)
-        vs = hv[:ns] if pairs else None
-        prm = oracle.Params(k=params["k"], a=30, M=M, k_policy=0 if params.get("k_policy") == "fixed" else 1,
-                            fill_div=4, seed=5489)
-        t0 = time.perf_counter()
-        oracle.sort(xs, vs, prm)
-        ct = time.perf_counter() - t0
-        cpu = {"value": ns / ct / 1e9, "unit": "Gkeys/s", "cores": 1, "kind": "oracle",
-               "sample": f"first {ns} keys of this workload's input, one oracle sort on one host thread ({ct:.1f} s)"}
+        cpu = cpu_baseline(wl, x, hv, params)
 
     if rank == 0:
         line = {

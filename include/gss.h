@@ -27,8 +27,11 @@
  *   - keys_in may equal keys_out (in place); vals_in may equal vals_out.
  *     Partial overlap, or temp overlapping an I/O buffer, is
  *     GSS_ERROR_INVALID_VALUE.
- *   - n == 0 succeeds without a launch.  n must be < 2^32 per call
- *     (u32 offsets), else GSS_ERROR_NOT_SUPPORTED.
+ *   - n == 0 succeeds without a launch.  Offsets are u32: a call needs
+ *     n + T < 2^32 (T = the tile) and n + 16*(n/(M+1) + 3) < 2^32 (per-bucket
+ *     16-aligned id ranges); with the default T and M that is about
+ *     n <= 2^32 - 2^19 - 2^16 for u64 keys.  Larger n returns
+ *     GSS_ERROR_NOT_SUPPORTED.
  *   - Errors are reported only through the return code: nothing aborts,
  *     throws or prints.  Asynchronous device faults surface at the
  *     caller's next synchronisation as usual in CUDA.

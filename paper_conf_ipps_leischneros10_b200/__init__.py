@@ -204,11 +204,25 @@ def _ptr(t):
     return None if t is None else ctypes.c_void_p(t.data_ptr())
 
 
-def _temp(fn, args_before_temp, stream_and_params, device):
+def _temp(fn, args_before_temp, stream_and_params, device, stream=None):
+    """Scratch of the size the C ABI asks for.  When the call runs on a stream
+    other than the current one, the scratch is recorded on that stream so the
+    caching allocator does not hand it out while the call's kernels run."""
     tb = _sz(0)
     _check(fn(*args_before_temp, None, ctypes.byref(tb), *stream_and_params), fn.__name__ + " (temp query)")
     temp = torch.empty(max(tb.value, 1), dtype=torch.uint8, device=device)
+    if isinstance(stream, torch.cuda.Stream):
+        temp.record_stream(stream)
     return temp, tb
+
+
+def _check_out(t: torch.Tensor | None, like: torch.Tensor, what: str):
+    """An output buffer must match its input in dtype, length and device and be contiguous."""
+    if t is None:
+        return
+    if t.dtype != like.dtype or t.numel() != like.numel() or t.device != like.device or not t.is_contiguous():
+        raise ValueError(f"{what} must be a contiguous {like.dtype} tensor of {like.numel()} elements on "
+                         f"{like.device}, got {t.dtype} x {t.numel()} on {t.device}")
 
 
 def sort(keys: torch.Tensor, values: torch.Tensor | None = None, *, out: torch.Tensor | None = None,
@@ -222,9 +236,15 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, *, out: torch.T
     lib = _lib()
     if not keys.is_cuda:
         raise ValueError("sort() takes CUDA tensors; use sort_host() for host buffers")
+    with torch.cuda.device(keys.device):
+        return _sort(lib, keys, values, out, values_out, descending, stats, profiler, stream, params)
+
+
+def _sort(lib, keys, values, out, values_out, descending, stats, profiler, stream, params):
     keys = keys.contiguous()
     kind = _kind(keys)
     n = keys.numel()
+    _check_out(out, keys, "out")
     out = torch.empty_like(keys) if out is None else out
     st = _Stats() if stats else None
     p = _params(stats=st, profiler=profiler, **params)
@@ -235,8 +255,9 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, *, out: torch.T
         if descending:
             raise NotImplementedError("descending order is exported for keys-only u64")
         values = values.contiguous()
-        if values.dtype != keys.dtype or values.numel() != n:
-            raise TypeError("values must have the key dtype and length")
+        if values.dtype != keys.dtype or values.numel() != n or values.device != keys.device:
+            raise TypeError("values must have the key dtype, length and device")
+        _check_out(values_out, values, "values_out")
         vout = torch.empty_like(values) if values_out is None else values_out
         fn = getattr(lib, f"gss_sort_pairs_{kind}")
         head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n)
@@ -249,7 +270,7 @@ def sort(keys: torch.Tensor, values: torch.Tensor | None = None, *, out: torch.T
         else:
             fn = getattr(lib, f"gss_sort_{kind}")
         head = (_ptr(keys), _ptr(out), n)
-    temp, tb = _temp(fn, head, (s, ctypes.byref(p)), keys.device)
+    temp, tb = _temp(fn, head, (s, ctypes.byref(p)), keys.device, stream)
     _check(fn(*head, _ptr(temp), ctypes.byref(tb), s, ctypes.byref(p)), fn.__name__)
     if stats:
         return out, vout, Stats._from(st)
@@ -387,20 +408,29 @@ def partition(keys: torch.Tensor, values: torch.Tensor | None = None, *, stream=
     lib = _lib()
     kind = _kind(keys)
     keys = keys.contiguous()
+    if values is not None:
+        values = values.contiguous()
+        if values.dtype != keys.dtype or values.numel() != keys.numel() or values.device != keys.device:
+            raise TypeError("values must have the key dtype, length and device")
     n = keys.numel()
     out = torch.empty_like(keys)
     vout = torch.empty_like(values) if values is not None else None
-    kcap = max(params.get("k") or 256, 4)
+    # k_b may exceed params['k'] only up to the ABI maximum: the default k is
+    # resolved from n inside the library (256 .. 1024), so size for 1024
+    kcap = 1024
     spl = torch.empty(kcap, dtype=keys.dtype, device=keys.device)
     off = torch.zeros(2 * kcap + 1, dtype=torch.uint64, device=keys.device)
     info = torch.zeros(4, dtype=torch.uint32, device=keys.device)
     p = _params(**params)
-    s = _stream(keys, stream)
-    fn = getattr(lib, f"gss_partition_{kind}")
-    head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n, _ptr(spl), _ptr(off), _ptr(info))
-    temp, tb = _temp(fn, head, (s, ctypes.byref(p)), keys.device)
-    _check(fn(*head, _ptr(temp), ctypes.byref(tb), s, ctypes.byref(p)), fn.__name__)
-    inf = [int(x) for x in info.cpu().tolist()]
+    with torch.cuda.device(keys.device):
+        s = _stream(keys, stream)
+        fn = getattr(lib, f"gss_partition_{kind}")
+        head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n, _ptr(spl), _ptr(off), _ptr(info))
+        temp, tb = _temp(fn, head, (s, ctypes.byref(p)), keys.device, stream)
+        _check(fn(*head, _ptr(temp), ctypes.byref(tb), s, ctypes.byref(p)), fn.__name__)
+        if isinstance(stream, torch.cuda.Stream):
+            stream.synchronize()
+        inf = [int(x) for x in info.cpu().tolist()]
     kb, ks, eq, K = inf
     return out, vout, spl[: max(ks - 1, 0)], off[: K + 1], tuple(inf)
 
@@ -411,18 +441,29 @@ def partition_by(keys: torch.Tensor, values: torch.Tensor | None, splitters: tor
     lib = _lib()
     kind = _kind(keys)
     keys = keys.contiguous()
+    if values is not None:
+        values = values.contiguous()
+        if values.dtype != keys.dtype or values.numel() != keys.numel() or values.device != keys.device:
+            raise TypeError("values must have the key dtype, length and device")
+    if splitters.dtype != keys.dtype or splitters.device != keys.device:
+        raise TypeError("splitters must have the key dtype and device")
+    spl = splitters.contiguous()          # kept alive until the call returns (and recorded on `stream`)
     n = keys.numel()
     out = torch.empty_like(keys)
     vout = torch.empty_like(values) if values is not None else None
-    nspl = splitters.numel()
+    nspl = spl.numel()
     counts = torch.zeros(nspl + 1, dtype=torch.uint64, device=keys.device)
-    s = _stream(keys, stream)
-    fn = getattr(lib, f"gss_partition_by_{kind}")
-    head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n, _ptr(splitters.contiguous()), nspl, _ptr(counts))
-    tb = _sz(0)
-    _check(fn(*head, None, ctypes.byref(tb), s), fn.__name__)
-    temp = torch.empty(max(tb.value, 1), dtype=torch.uint8, device=keys.device)
-    _check(fn(*head, _ptr(temp), ctypes.byref(tb), s), fn.__name__)
+    with torch.cuda.device(keys.device):
+        s = _stream(keys, stream)
+        fn = getattr(lib, f"gss_partition_by_{kind}")
+        head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n, _ptr(spl), nspl, _ptr(counts))
+        tb = _sz(0)
+        _check(fn(*head, None, ctypes.byref(tb), s), fn.__name__)
+        temp = torch.empty(max(tb.value, 1), dtype=torch.uint8, device=keys.device)
+        if isinstance(stream, torch.cuda.Stream):
+            temp.record_stream(stream)
+            spl.record_stream(stream)
+        _check(fn(*head, _ptr(temp), ctypes.byref(tb), s), fn.__name__)
     return out, vout, counts
 
 

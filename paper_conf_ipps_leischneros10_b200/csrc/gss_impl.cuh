@@ -7,6 +7,7 @@
 // in-SM sorts, largest size class first, copy, overflow) on the
 // caller's stream; all data-dependent work lists live in device memory.
 #include <algorithm>
+#include <atomic>
 #include <cstdio>
 #include <cstring>
 #include <mutex>
@@ -228,6 +229,14 @@ gss_status set_smem(K kernel, size_t bytes) {
   return GSS_SUCCESS;
 }
 
+// Per-device cache of a grid size (the occupancy query costs host time on
+// launch-bound sorts).  Racing threads store the same value.
+struct GridCache {
+  std::atomic<int> g[64];
+  int get(int dev) const { return dev >= 0 && dev < 64 ? g[dev].load(std::memory_order_relaxed) : 0; }
+  void put(int dev, int v) { if (dev >= 0 && dev < 64) g[dev].store(v, std::memory_order_relaxed); }
+};
+
 template <class K>
 int grid_for(K kernel, int threads, size_t smem, int sms, int cap = 1 << 30) {
   int per = 0;
@@ -298,17 +307,17 @@ struct Engine {
       const int ns = std::min(nt, kSplitMaxThreads);
       const size_t smem = small_smem_bytes<Key, Val>(cfg.class_cap[cls]);
       GSS_TRY(set_smem(kern, small_smem_bytes<Key, Val>(cfg.class_cap[kNumClasses - 1])));
-      static int grid[kNumClasses] = {};
-      if (!grid[cls]) grid[cls] = grid_for(kern, ns, smem, di.sms);
-      const int g = grid[cls];
+      static GridCache grid[kNumClasses];
+      int g = grid[cls].get(di.dev);
+      if (!g) { g = grid_for(kern, ns, smem, di.sms); grid[cls].put(di.dev, g); }
       return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, ns, smem, s>>>(c, (uint32_t)cls); });
     }
     auto kern = k_small_block<Key, Val, IdT, Cmp>;
     const size_t smem = block_sort_smem_bytes<Key, Val>(nt);
     GSS_TRY(set_smem(kern, block_sort_smem_bytes<Key, Val>(kSmallMaxThreads)));
-    static int grid[kNumClasses + 1] = {};
-    if (!grid[cls]) grid[cls] = grid_for(kern, nt, smem, di.sms);
-    const int g = grid[cls];
+    static GridCache grid[kNumClasses + 1];
+    int g = grid[cls].get(di.dev);
+    if (!g) { g = grid_for(kern, nt, smem, di.sms); grid[cls].put(di.dev, g); }
     return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, nt, smem, s>>>(c, (uint32_t)cls); });
   }
 
@@ -328,9 +337,10 @@ struct Engine {
     GSS_TRY(set_smem(ks, sm_sample));
     GSS_TRY(set_smem(kc, sm_cls));
     GSS_TRY(set_smem(ksc, sm_sc));
-    static int g_sample = 0, g_plan = 0;
-    if (!g_sample) g_sample = grid_for(ks, kSampleThreads, sm_sample, di.sms);
-    if (!g_plan) g_plan = grid_for(k_plan<Key, Val, IdT>, kPlanThreads, 0, di.sms);
+    static GridCache gc_sample, gc_plan;
+    int g_sample = gc_sample.get(di.dev), g_plan = gc_plan.get(di.dev);
+    if (!g_sample) { g_sample = grid_for(ks, kSampleThreads, sm_sample, di.sms); gc_sample.put(di.dev, g_sample); }
+    if (!g_plan) { g_plan = grid_for(k_plan<Key, Val, IdT>, kPlanThreads, 0, di.sms); gc_plan.put(di.dev, g_plan); }
     const int g_cls = grid_for(kc, kClsThreads, sm_cls, di.sms);
     const int g_sc = grid_for(ksc, kScatterThreads, sm_sc, di.sms);
     auto ksf = k_scatter_fast<Key, Val, IdT, Cmp>;
@@ -470,6 +480,9 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
     using IdT = decltype(id_tag);
     Layout<Key, Val, IdT> lay;
     lay.compute(n, cfg, mode, host_io);
+    // every element offset, tile start and 16-aligned id offset is a u32
+    if ((uint64_t)n + cfg.T >= (1ull << 32) || (uint64_t)n + 16ull * ((uint64_t)lay.cap_buckets + 2) >= (1ull << 32))
+      return GSS_ERROR_NOT_SUPPORTED;
     if (!temp) { *temp_bytes = lay.total; return GSS_SUCCESS; }
     if (*temp_bytes < lay.total) return GSS_ERROR_TEMP_TOO_SMALL;
     if (n == 0) {

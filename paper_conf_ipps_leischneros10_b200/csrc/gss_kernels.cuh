@@ -81,7 +81,7 @@ __global__ void k_init(Ctx<Key, Val, IdT> c) {
   } else {
     kb = choose_kb(c.k, c.k_policy, c.fill_div, c.M, c.n);
   }
-  uint32_t nt = (c.n + c.T - 1) / c.T;
+  uint32_t nt = (uint32_t)(((uint64_t)c.n + c.T - 1) / c.T);
   Bucket B{};
   B.lo = 0; B.m = c.n; B.tile_start = 0; B.ntiles = nt; B.kb = kb;
   B.hist_base = 0; B.spl_base = 0; B.id_base = 0;
@@ -1251,7 +1251,7 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
         }
       }
       if (__any_sync(kFull, to_copy)) {
-        const uint32_t nt = to_copy ? (m + c.T - 1) / c.T : 0;
+        const uint32_t nt = to_copy ? (uint32_t)(((uint64_t)m + c.T - 1) / c.T) : 0;
         const uint32_t i = warp_append(&c.cnt->copy_count, nt);
         if (to_copy) {
           if (i + nt <= c.cap_copy) {
@@ -1264,7 +1264,7 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
       if (__any_sync(kFull, to_next)) {
         LevelCounters& NL = c.cnt->lvl[next];
         const uint32_t kb = to_next ? choose_kb(c.k, c.k_policy, c.fill_div, c.M, m) : 0;
-        const uint32_t nt = to_next ? (m + c.T - 1) / c.T : 0;
+        const uint32_t nt = to_next ? (uint32_t)(((uint64_t)m + c.T - 1) / c.T) : 0;
         const uint32_t bi = warp_append(&NL.num_buckets, to_next ? 1u : 0u);
         const uint32_t ts = warp_append(&NL.num_tiles, nt);
         const uint32_t hbn = warp_append(&NL.hist_alloc, to_next ? max(kb, 3u) * nt : 0u);

@@ -5,6 +5,8 @@ same multiset of (key, value) pairs; one distribution level (gss_partition)
 must equal the oracle's stable partition, splitters and bucket sizes
 bit-exact (R7).
 """
+import os
+
 import numpy as np
 import pytest
 import torch
@@ -31,9 +33,12 @@ def to_host(t: torch.Tensor) -> np.ndarray:
     return t.cpu().numpy()
 
 
-def oracle_params(oracle_mod, k=256, M=16384, a=30, seed=5489, k_policy="adaptive", fill_div=4):
+NPROC = os.cpu_count() or 1
+
+
+def oracle_params(oracle_mod, k=256, M=16384, a=30, seed=5489, k_policy="adaptive", fill_div=4, threads=NPROC):
     return oracle_mod.Params(k=k, a=a, M=M, k_policy=1 if k_policy == "adaptive" else 0, fill_div=fill_div,
-                             sample_cap=16384, seed=seed)
+                             sample_cap=16384, seed=seed, threads=threads)
 
 
 def _few(n, width):
@@ -315,30 +320,113 @@ def test_distributed_sorter_single_rank_nccl(gss):
 
 
 @pytest.mark.parametrize("width,pairs", KINDS)
-def test_stable_flag_same_keys(gss, width, pairs):
-    """GSS_FLAG_STABLE (ballot-ranked stable scatter) and the default atomic-ranked scatter agree on keys."""
+def test_stable_flag_same_keys(gss, oracle_mod, width, pairs):
+    """GSS_FLAG_STABLE (ballot-ranked stable scatter) and the default atomic-ranked scatter
+    both give the oracle's keys; the level structure matches the oracle's records."""
     n = (1 << 20) + 3
     x = inputs.keys("and2", n, width, seed=4)
     v = inputs.values(n, width) if pairs else None
-    a = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=4)
-    b = gss.sort(to_dev(x), to_dev(v) if pairs else None)
-    np.testing.assert_array_equal(to_host(a[0]), to_host(b[0]))
-    np.testing.assert_array_equal(to_host(a[0]), np.sort(x))
-    if pairs:
-        check_pairs(x, to_host(a[1]), np.sort(x))
-        check_pairs(x, to_host(b[1]), np.sort(x))
+    M = 4096
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=M, threads=NPROC), log=True)
+    for flags in (4, 0):
+        ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=M, flags=flags, stats=True)
+        np.testing.assert_array_equal(to_host(ko), ok)
+        if pairs:
+            check_pairs(x, to_host(vo), ok)
+        assert_levels_match(st, recs)
 
 
 @pytest.mark.parametrize("width,pairs", KINDS)
-def test_direct_scatter_ablation(gss, width, pairs):
-    """GSS_FLAG_DIRECT_SCATTER (the paper's unstructured Phase 4) sorts correctly."""
+def test_direct_scatter_ablation(gss, oracle_mod, width, pairs):
+    """GSS_FLAG_DIRECT_SCATTER (the paper's unstructured Phase 4) gives the oracle's keys."""
     n = (1 << 20) + 11
     x = inputs.keys("staggered", n, width, seed=3)
     v = inputs.values(n, width) if pairs else None
-    ko, vo = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=8)
-    np.testing.assert_array_equal(to_host(ko), np.sort(x))
+    M = 4096
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=M, threads=NPROC), log=True)
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=M, flags=8, stats=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
     if pairs:
-        check_pairs(x, to_host(vo), np.sort(x))
+        check_pairs(x, to_host(vo), ok)
+    assert_levels_match(st, recs)
+
+
+# ---------------------------------------------------------------------------
+# The configuration bench.py times: library defaults (auto k = 256, auto tile
+# T = 65536 so every tile spans 16 scatter chunks, M = the in-SM capacity),
+# the persistent grids walking hundreds of tiles, and the CUDA-graph replay
+# (GSS_FLAG_GRAPH) -- element by element against the oracle.
+# ---------------------------------------------------------------------------
+def default_M(width, pairs):
+    return 8192 if (pairs and width == 64) else (32768 if (width == 32 and not pairs) else 16384)
+
+
+def default_k(n, M):
+    k = 256
+    while k < 1024 and n > k * k * (M // 2):
+        k *= 2
+    return k
+
+
+def assert_levels_match(st, recs):
+    for lvl in range(4):
+        assert st.split_elems[lvl] == sum(r.m for r in recs if r.level == lvl), (lvl, st.split_elems[:4])
+    assert st.overflow_buckets == 0 and st.error_flags == 0
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist", ["uniform", "dd", "and4", "sorted"])
+def test_bench_config_parity(gss, oracle_mod, width, pairs, dist):
+    n = (1 << 25) + 777                                     # 513 tiles of 65536 keys, ragged last tile
+    x = inputs.keys(dist, n, width, seed=1)
+    v = inputs.values(n, width) if pairs else None
+    M = default_M(width, pairs)
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, k=default_k(n, M), M=M, threads=NPROC),
+                                  log=True)
+    # library defaults, with statistics (direct launches)
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, stats=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if pairs:
+        check_pairs(x, to_host(vo), ok)
+    assert_levels_match(st, recs)
+    # the bench's path: a persistent Sorter with the CUDA-graph flag; the second
+    # call replays the captured graph
+    kind = f"u{width}"
+    s = gss.Sorter(kind, n, pairs, flags=16)
+    kin, kout = to_dev(x), torch.empty(n, dtype=DT[width], device="cuda")
+    vin = to_dev(v) if pairs else None
+    vout = torch.empty_like(vin) if pairs else None
+    for _ in range(2):
+        kout.zero_()
+        s(kin, kout, vin, vout)
+    np.testing.assert_array_equal(to_host(kout), ok)
+    if pairs:
+        check_pairs(x, to_host(vout), ok)
+
+
+@pytest.mark.parametrize("width,n,pairs,dist", [(64, 1 << 28, False, "uniform"), (64, 1 << 27, True, "uniform"),
+                                                (64, 1 << 27, True, "and4"), (32, 1 << 27, False, "staggered")])
+def test_full_size_elementwise(gss, oracle_mod, width, n, pairs, dist):
+    """BASELINE configs[1-3] sizes (2^28 u64 is the north-star row) through the
+    bench's Sorter + graph path, compared element by element with the oracle."""
+    x = inputs.keys(dist, n, width, seed=1)
+    v = inputs.values(n, width) if pairs else None
+    M = default_M(width, pairs)
+    s = gss.Sorter(f"u{width}", n, pairs, flags=16)
+    kin = to_dev(x)
+    kout = torch.empty_like(kin)
+    vin = to_dev(v) if pairs else None
+    vout = torch.empty_like(vin) if pairs else None
+    for _ in range(2):
+        s(kin, kout, vin, vout)
+    got = to_host(kout)
+    gv = to_host(vout) if pairs else None
+    del kin, kout, vin, vout
+    torch.cuda.empty_cache()
+    ok, _, _ = oracle_mod.sort(x, None, oracle_params(oracle_mod, k=default_k(n, M), M=M, threads=NPROC))
+    np.testing.assert_array_equal(got, ok)
+    if pairs:
+        check_pairs(x, gv, ok)
 
 
 def test_graph_replay(gss):
