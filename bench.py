@@ -278,20 +278,16 @@ def run_reference(args, wl):
 # ---------------------------------------------------------------------------
 # our arm
 # ---------------------------------------------------------------------------
-def run_ours(args, wl):
+def run_single(args, wl):
     os.environ.setdefault("NCCL_DEBUG", "WARN")          # keep stdout to the one JSON line
     import torch
     import torch.distributed as dist_mod
 
     import paper_conf_ipps_leischneros10_b200 as gss
 
-    world = int(os.environ.get("WORLD_SIZE", "1"))
-    rank = int(os.environ.get("RANK", "0"))
-    local = int(os.environ.get("LOCAL_RANK", "0"))
+    world, rank, local = 1, 0, int(os.environ.get("LOCAL_RANK", "0"))
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
-    if world > 1:
-        dist_mod.init_process_group("nccl", device_id=dev)
 
     n, bits, pairs, distname, desc = WORKLOADS[wl]
     wk = bits // 8
@@ -307,20 +303,11 @@ def run_ours(args, wl):
     dvals = torch.from_numpy(hv).to(dev) if pairs else None
     stream = torch.cuda.current_stream(dev)
 
-    use_dist = world > 1 or args.force_dist
-    if use_dist:
-        if world == 1 and not dist_mod.is_initialized():
-            os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
-            os.environ.setdefault("MASTER_PORT", "29533")
-            dist_mod.init_process_group("nccl", rank=0, world_size=1, device_id=dev)
-        from paper_conf_ipps_leischneros10_b200 import dist as gdist
-        sorter = gdist.DistSorter(kind, n, pairs, device=dev, **params)
-        step = lambda: sorter(dkeys, dvals)  # noqa: E731
-    else:
-        sorter = gss.Sorter(kind, n, pairs, device=dev, **params)
-        kout = torch.empty_like(dkeys)
-        vout = torch.empty_like(dvals) if pairs else None
-        step = lambda: sorter(dkeys, kout, dvals, vout)  # noqa: E731
+    use_dist = False
+    sorter = gss.Sorter(kind, n, pairs, device=dev, **params)
+    kout = torch.empty_like(dkeys)
+    vout = torch.empty_like(dvals) if pairs else None
+    step = lambda: sorter(dkeys, kout, dvals, vout)  # noqa: E731
 
     for _ in range(args.warmup):
         step()
@@ -341,29 +328,18 @@ def run_ours(args, wl):
         torch.cuda.synchronize(dev)
         barrier()
     ms = e0.elapsed_time(e1) / args.steps
-    if world > 1:
-        t = torch.tensor([ms], device=dev, dtype=torch.float64)
-        dist_mod.all_reduce(t, op=dist_mod.ReduceOp.MAX)
-        ms = float(t.item())
     value = n * world / (ms * 1e-3) / 1e9
 
     # ---- result check (not timed) ----
-    if not use_dist:
-        ok = mix_check(x, kout.cpu().numpy())
-        if pairs:
-            ok = ok and pairs_check(x, kout.cpu().numpy(), vout.cpu().numpy(), rank * n)
-    else:
-        ok = sorter.verify(x)
+    ok = mix_check(x, kout.cpu().numpy())
+    if pairs:
+        ok = ok and pairs_check(x, kout.cpu().numpy(), vout.cpu().numpy(), rank * n)
 
     # ---- per-kernel breakdown (separate profiled steps, CUDA events per launch) ----
     extra = {}
     roof = None
     gpu_launches = None
     hbm, peak_src = peaks()
-    if use_dist:
-        gpu_launches = sorter.count_launches(dkeys, dvals) * args.steps
-        extra["exchange"] = {"send_counts": sorter.last_counts[0], "recv_counts": sorter.last_counts[1],
-                             "samples_per_rank": sorter.S}
     if not use_dist:
         st = sorter(dkeys, kout, dvals, vout, stats=True)
         gpu_launches = st.launches * args.steps
@@ -422,7 +398,7 @@ def run_ours(args, wl):
 
     # ---- CPU baseline: the oracle on a bounded sample (rank 0, N == 1 only) ----
     cpu = None
-    if world == 1 and not use_dist and not args.no_cpu_baseline:
+    if not args.no_cpu_baseline:
         cpu = cpu_baseline(wl, x, hv, params)
 
     if rank == 0:
@@ -436,9 +412,170 @@ def run_ours(args, wl):
             "clocks": clk.summary(), "result_check": bool(ok), **extra,
         }
         print(json.dumps(line), flush=True)
-    if dist_mod.is_initialized():
-        dist_mod.destroy_process_group()
     return 0 if ok else 1
+
+NVLINK_GBS = 770.0   # measured peer copy per direction (B200_PROFILING.md; 900 nominal)
+
+
+def run_dist(args, wl):
+    """N > 1 (or --force-dist): the distributed sample sort (gss_dist_*, NCCL
+    over NVLink), weak scaling: n keys per GPU, n*N in total.  Device time of
+    K calls on every rank (barrier + synchronize on both sides), max over ranks."""
+    import torch
+    import torch.distributed as dist_mod
+
+    import paper_conf_ipps_leischneros10_b200 as gss
+    from paper_conf_ipps_leischneros10_b200 import dist as gdist
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if not dist_mod.is_initialized():
+        os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        os.environ.setdefault("MASTER_PORT", "29533")
+        dist_mod.init_process_group("nccl", rank=rank, world_size=world, device_id=dev)
+
+    n, bits, pairs, distname, desc = WORKLOADS[wl]
+    wk = bits // 8
+    wv = wk if pairs else 0
+    kind = f"u{bits}"
+    params = workload_params(wl)
+    params.pop("flags", None)                  # no graph replay: the received count varies per call
+    x = inputs.keys(distname, n * world, bits, seed=1, start=rank * n, count=n)
+    hv = inputs.values(n, bits, start=rank * n) if pairs else None
+    dkeys = torch.from_numpy(x).to(dev)
+    dvals = torch.from_numpy(hv).to(dev) if pairs else None
+    stream = torch.cuda.current_stream(dev)
+    sorter = gdist.DistSorter(kind, n, pairs, device=dev, **params)
+    step = lambda: sorter(dkeys, dvals)  # noqa: E731
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize(dev)
+
+    def max_over_ranks(v):
+        t = torch.tensor([v], device=dev, dtype=torch.float64)
+        dist_mod.all_reduce(t, op=dist_mod.ReduceOp.MAX)
+        return float(t.item())
+
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    with ClockSampler(local) as clk:
+        dist_mod.barrier()
+        torch.cuda.synchronize(dev)
+        e0.record(stream)
+        for _ in range(args.steps):
+            step()
+        e1.record(stream)
+        torch.cuda.synchronize(dev)
+        dist_mod.barrier()
+    ms = max_over_ranks(e0.elapsed_time(e1) / args.steps)
+    value = n * world / (ms * 1e-3) / 1e9
+    ok = sorter.verify(x, hv)
+    send, recv, cuts = sorter.last_exchange()
+
+    # per-kernel breakdown of our kernels inside the call (CUDA events per launch) and the roofline
+    hbm, peak_src = peaks()
+    prof = gss.Profiler()
+    kp = max(3, min(args.steps, 5))
+    st = None
+    for i in range(kp):
+        r = sorter(dkeys, dvals, profiler=prof, stats=(i == 0))
+        if i == 0:
+            st = r[3]
+    torch.cuda.synchronize(dev)
+    per = {k: (v[0] / kp, v[1] / kp) for k, v in prof.read().items() if v[1]}
+    launches = int(round(sum(v[1] for v in per.values()))) + 1 + (1 if world > 1 else 0)   # + sample, splitter pick
+    n_recv = sorter.n_out
+    # algorithmic bytes: global level (classify w_k, scatter 2(w_k+w_v) over n) + the local sort's levels
+    # and in-SM sort (from its statistics) + the all-to-all bytes that leave this GPU over NVLink
+    local_sort_B = total_alg_bytes(st, wk, wv, params["k"], params["tile"], params["a"])
+    B_local = n * (3 * wk + 2 * wv) + local_sort_B
+    B_a2a = sum(c for q, c in enumerate(send) if q != rank) * (wk + wv)
+    t_roof = B_local / (hbm * 1e9) + B_a2a / (NVLINK_GBS * 1e9)
+    t_roof = max_over_ranks(t_roof)
+    dom = max(per, key=lambda k: per[k][0])
+    roof = {"bound": "hbm+nvlink", "kernel": dom, "achieved": None, "peak": hbm, "unit": "GB/s",
+            "frac": round(t_roof / (ms * 1e-3), 4), "traffic": None, "t_roof_ms": t_roof * 1e3,
+            "alg_bytes_local": B_local, "a2a_bytes_out": B_a2a, "nvlink_gbs": NVLINK_GBS, "peak_source": peak_src,
+            "note": "frac = (B_local / HBM + B_a2a / NVLink) / measured step time (SURVEY 8(d) d.6), max over ranks"}
+    if dom in ("classify", "scatter", "small_sort"):
+        # the dominant kernel kind summed over the global partition and the local sort
+        ab = {"classify": (n + sum(st.split_elems)) * wk,
+              "scatter": (n + sum(st.split_elems)) * 2 * (wk + wv),
+              "small_sort": st.small_elems * 2 * (wk + wv)}[dom]
+        roof["achieved"] = round(ab / (per[dom][0] * 1e-3) / 1e9, 1)
+        roof["kernel_frac"] = round(roof["achieved"] / hbm, 4)
+
+    # end to end: pinned host shard -> device, distributed sort, received range -> host, every step
+    hk = torch.from_numpy(x).pin_memory()
+    hvi = torch.from_numpy(hv).pin_memory() if pairs else None
+    hko = torch.empty(sorter.capacity, dtype=dkeys.dtype).pin_memory()
+    hvo = torch.empty(sorter.capacity, dtype=dkeys.dtype).pin_memory() if pairs else None
+    ke = max(3, min(args.steps, 5))
+    dist_mod.barrier()
+    torch.cuda.synchronize(dev)
+    e0.record(stream)
+    d2h = 0
+    for _ in range(ke):
+        dkeys.copy_(hk, non_blocking=True)
+        if pairs:
+            dvals.copy_(hvi, non_blocking=True)
+        k, v, nr = sorter(dkeys, dvals)
+        hko[:nr].copy_(k, non_blocking=True)
+        if pairs:
+            hvo[:nr].copy_(v, non_blocking=True)
+        d2h = nr * (wk + wv)
+    e1.record(stream)
+    torch.cuda.synchronize(dev)
+    ems = max_over_ranks(e0.elapsed_time(e1) / ke)
+    e2e = {"value": n * world / (ems * 1e-3) / 1e9, "unit": "Gkeys/s", "h2d_bytes_per_step": n * (wk + wv),
+           "d2h_bytes_per_step": d2h, "ms_per_step": ems,
+           "path": "DistSorter (gss_dist_sort_*): pinned host shard H2D, distributed sort, received range D2H"}
+    okt = torch.tensor([1 if ok else 0], device=dev)
+    dist_mod.all_reduce(okt, op=dist_mod.ReduceOp.MIN)
+    ok = bool(okt.item())
+    if rank == 0:
+        line = {
+            "metric": metric_name(pairs),
+            "value": round(value, 3), "unit": "Gkeys/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": round(ms, 4), "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": kind, "data": "synthetic",
+            "config": {**config_dict(wl, world, params), "path": "gss_dist_sort (NCCL all-to-all-v)",
+                       "n_total": n * world},
+            "roofline": roof, "cpu_baseline": None, "e2e": e2e, "gpu_launches": launches * args.steps,
+            "clocks": clk.summary(), "result_check": ok,
+            "exchange": {"send_counts_rank0": send, "recv_counts_rank0": recv, "cuts": cuts,
+                         "n_recv_rank0": n_recv},
+            "kernels_ms_per_step_rank0": {k: round(v[0], 4) for k, v in per.items()},
+        }
+        print(json.dumps(line), flush=True)
+    del sorter
+    dist_mod.destroy_process_group()
+    return 0 if ok else 1
+
+
+def spawn_ranks(args) -> int:
+    """`python bench.py --gpus N` without torchrun: launch N ranks (one process per GPU) through
+    torch.distributed.run on this node and pass their output through."""
+    import socket
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
+           "--master-addr", "127.0.0.1", "--master-port", str(port), os.path.abspath(__file__), *sys.argv[1:]]
+    return subprocess.call(cmd)
+
+
+def run_ours(args, wl):
+    os.environ.setdefault("NCCL_DEBUG", "WARN")          # keep stdout to the one JSON line
+    world = int(os.environ.get("WORLD_SIZE", "0"))
+    if world == 0 and args.gpus > 1:
+        return spawn_ranks(args)
+    if max(world, 1) > 1 or args.force_dist:
+        return run_dist(args, wl)
+    return run_single(args, wl)
 
 
 def main():

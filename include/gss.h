@@ -237,6 +237,71 @@ gss_status gss_partition_by_u64(const uint64_t* keys_in, const uint64_t* vals_in
                                 const uint64_t* splitters, uint32_t nspl, uint64_t* counts_out,
                                 void* temp, size_t* temp_bytes, void* stream);
 
+/* The same in equality mode (R4 applied to given splitters; the global level
+ * of gss_dist_sort_*): key e gets id 2b (range: spl[b-1] < e < spl[b]) or
+ * 2b+1 (e == spl[b]) with b = #{spl < e}; counts_out holds 2*nspl+1 sizes.
+ * Duplicate splitters are allowed (every copy of a key lands in one
+ * equality bucket).  nspl <= 127. */
+gss_status gss_partition_by_eq_u32(const uint32_t* keys_in, const uint32_t* vals_in,
+                                   uint32_t* keys_out, uint32_t* vals_out, size_t n,
+                                   const uint32_t* splitters, uint32_t nspl, uint64_t* counts_out,
+                                   void* temp, size_t* temp_bytes, void* stream);
+gss_status gss_partition_by_eq_u64(const uint64_t* keys_in, const uint64_t* vals_in,
+                                   uint64_t* keys_out, uint64_t* vals_out, size_t n,
+                                   const uint64_t* splitters, uint32_t nspl, uint64_t* counts_out,
+                                   void* temp, size_t* temp_bytes, void* stream);
+
+/* ---------------------------------------------------------------------- */
+/* Distributed sample sort across GPUs: one process per GPU, NCCL over     */
+/* NVLink (sample sort's home is distributed memory, */
+/* P:195-196; large random samples balance the parts).          */
+/* Each rank passes its shard keys_in[0..n_local); on return rank r holds  */
+/* the r-th contiguous range of the global sorted order in                 */
+/* keys_out[0..*n_out) (values with their keys).  Steps: all-gather of      */
+/* (n_local, out_capacity); 16384 hashed samples per rank (level tag 255,  */
+/* lo = the shard's global start, R2), all-gathered and sorted identically */
+/* on every rank; P-1 splitters S[(i+1)VS/P - 1] (R1); equality-mode       */
+/* partition (gss_partition_by_eq); all-gather of the 2P-1 counts; the      */
+/* exchange plan gss_dist_plan; grouped ncclSend/ncclRecv (all-to-all-v);   */
+/* in-place gss_sort of the received range.  Two host synchronisations per */
+/* call (the two small all-gathers).  temp == NULL queries *temp_bytes     */
+/* (depends on n_local and out_capacity; no GPU or NCCL access).            */
+/* Errors: GSS_ERROR_NCCL (a collective failed), GSS_ERROR_CAPACITY (some  */
+/* rank's out_capacity is below what it would receive: every rank returns  */
+/* it, nothing is exchanged, *n_out = this rank's required count).  A      */
+/* handle is not thread-safe; all ranks must call collectively.            */
+/* ---------------------------------------------------------------------- */
+typedef struct gss_dist gss_dist;
+/* rank 0 creates the id and shares it (e.g. torch.distributed broadcast) */
+gss_status gss_dist_unique_id(uint8_t id_out[128]);
+gss_status gss_dist_create(gss_dist** d, const uint8_t id[128], int rank, int nranks, int device);
+gss_status gss_dist_destroy(gss_dist* d);
+gss_status gss_dist_sort_u32(gss_dist* d, const uint32_t* keys_in, size_t n_local, uint32_t* keys_out,
+                             size_t out_capacity, size_t* n_out /* host */, void* temp, size_t* temp_bytes,
+                             void* stream, const gss_params* p);
+gss_status gss_dist_sort_u64(gss_dist* d, const uint64_t* keys_in, size_t n_local, uint64_t* keys_out,
+                             size_t out_capacity, size_t* n_out, void* temp, size_t* temp_bytes,
+                             void* stream, const gss_params* p);
+gss_status gss_dist_sort_pairs_u32(gss_dist* d, const uint32_t* keys_in, const uint32_t* vals_in, size_t n_local,
+                                   uint32_t* keys_out, uint32_t* vals_out, size_t out_capacity, size_t* n_out,
+                                   void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+gss_status gss_dist_sort_pairs_u64(gss_dist* d, const uint64_t* keys_in, const uint64_t* vals_in, size_t n_local,
+                                   uint64_t* keys_out, uint64_t* vals_out, size_t out_capacity, size_t* n_out,
+                                   void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
+/* The last call's plan on this rank: P send counts, P receive counts, P+1 cuts (host arrays, may be NULL). */
+gss_status gss_dist_last_exchange(const gss_dist* d, uint64_t* send_counts, uint64_t* recv_counts, uint64_t* cuts);
+
+/* The exchange plan (host only, no GPU): counts[q*K + i] = rank q's number of
+ * keys with global-level id i (K = 2P-1; even ids are range buckets, which
+ * stay whole, odd ids equality buckets, whose keys are all equal and may be
+ * split).  Rank q owns global positions [cuts[q], cuts[q+1]) of the order
+ * (bucket, source rank, position): each cut is the balanced target q*N/P,
+ * moved to the nearer boundary when it falls inside a range bucket.  For
+ * rank `me`: send_off/send_cnt[q] = the range of its partitioned shard that
+ * goes to rank q; recv_cnt[q] = what it receives from rank q. */
+gss_status gss_dist_plan(uint32_t P, uint32_t me, uint32_t K, const uint64_t* counts, uint64_t* cuts,
+                         uint64_t* send_off, uint64_t* send_cnt, uint64_t* recv_cnt);
+
 /* ---------------------------------------------------------------------- */
 /* Profiling: CUDA events around every launch of the calls that carry the */
 /* profiler in their params.  Read after the stream has been synchronised. */

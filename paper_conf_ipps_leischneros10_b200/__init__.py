@@ -99,7 +99,8 @@ def _lib():
             f = getattr(lib, name)
             f.restype = ctypes.c_int
             f.argtypes = [_vp, _vp, _vp, _vp, _sz, _vp, _vp, _vp, _vp, szp, _vp, P]
-        for name in ("gss_partition_by_u32", "gss_partition_by_u64"):
+        for name in ("gss_partition_by_u32", "gss_partition_by_u64", "gss_partition_by_eq_u32",
+                     "gss_partition_by_eq_u64"):
             f = getattr(lib, name)
             f.restype = ctypes.c_int
             f.argtypes = [_vp, _vp, _vp, _vp, _sz, _vp, _u32, _vp, _vp, szp, _vp]
@@ -435,9 +436,11 @@ def partition(keys: torch.Tensor, values: torch.Tensor | None = None, *, stream=
     return out, vout, spl[: max(ks - 1, 0)], off[: K + 1], tuple(inf)
 
 
-def partition_by(keys: torch.Tensor, values: torch.Tensor | None, splitters: torch.Tensor, *, stream=None):
+def partition_by(keys: torch.Tensor, values: torch.Tensor | None, splitters: torch.Tensor, *, stream=None,
+                 eq: bool = False):
     """Stable partition of keys into len(splitters)+1 buckets by given sorted
-    splitters (ties go left).  Returns (keys_out, values_out, counts[u64])."""
+    splitters (ties go left).  Returns (keys_out, values_out, counts[u64]).
+    eq=True: equality mode (R4), 2*len(splitters)+1 buckets (gss_partition_by_eq)."""
     lib = _lib()
     kind = _kind(keys)
     keys = keys.contiguous()
@@ -452,10 +455,10 @@ def partition_by(keys: torch.Tensor, values: torch.Tensor | None, splitters: tor
     out = torch.empty_like(keys)
     vout = torch.empty_like(values) if values is not None else None
     nspl = spl.numel()
-    counts = torch.zeros(nspl + 1, dtype=torch.uint64, device=keys.device)
+    counts = torch.zeros(2 * nspl + 1 if eq else nspl + 1, dtype=torch.uint64, device=keys.device)
     with torch.cuda.device(keys.device):
         s = _stream(keys, stream)
-        fn = getattr(lib, f"gss_partition_by_{kind}")
+        fn = getattr(lib, f"gss_partition_by_{'eq_' if eq else ''}{kind}")
         head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n, _ptr(spl), nspl, _ptr(counts))
         tb = _sz(0)
         _check(fn(*head, None, ctypes.byref(tb), s), fn.__name__)

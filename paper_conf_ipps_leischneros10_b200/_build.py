@@ -23,6 +23,19 @@ FLAGS = ARCH + ["-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr", "-
                 "-Xptxas", "-v"] + os.environ.get("GSS_NVCC_EXTRA", "").split()   # tuning experiments (-D...)
 
 
+def nccl_dirs():
+    """The NCCL that torch ships (2.28.x: nccl.h + libnccl.so.2); libgss.so links it with an rpath so the
+    process shares torch's copy."""
+    try:
+        import nvidia.nccl as nn
+        base = list(nn.__path__)[0]
+    except Exception:  # pragma: no cover - image without the wheel
+        base = None
+    if base and os.path.exists(os.path.join(base, "include", "nccl.h")):
+        return os.path.join(base, "include"), os.path.join(base, "lib")
+    return "/usr/include", "/usr/lib/x86_64-linux-gnu"
+
+
 def sources():
     return sorted(glob.glob(os.path.join(CSRC, "*.cu")))
 
@@ -40,7 +53,8 @@ def stale() -> bool:
 
 def _compile(src: str):
     obj = os.path.join(OBJ, os.path.basename(src)[:-3] + ".o")
-    cmd = [NVCC, *FLAGS, "-c", "-o", obj, src]
+    inc, _ = nccl_dirs()
+    cmd = [NVCC, *FLAGS, "-I", inc, "-c", "-o", obj, src]
     r = subprocess.run(cmd, capture_output=True, text=True)
     return src, obj, cmd, r
 
@@ -60,7 +74,9 @@ def build(force: bool = False, verbose: bool = False) -> str:
     if bad:
         sys.stderr.write(bad[0][3].stderr[-4000:])
         raise RuntimeError(f"nvcc failed for {[os.path.basename(b[0]) for b in bad]}; see {log}")
-    cmd = [NVCC, *ARCH, "-shared", "-o", LIB + ".tmp", *[r[1] for r in results]]
+    _, libdir = nccl_dirs()
+    cmd = [NVCC, *ARCH, "-shared", "-o", LIB + ".tmp", *[r[1] for r in results], "-L", libdir, "-l:libnccl.so.2",
+           "-Xlinker", f"-rpath,{libdir}"]
     r = subprocess.run(cmd, capture_output=True, text=True)
     with open(log, "a") as f:
         f.write(" ".join(cmd) + "\n" + r.stdout + r.stderr)

@@ -235,7 +235,7 @@ gss_status gss_partition_by_u32(const uint32_t* ki, const uint32_t* vi, uint32_t
                                 const uint32_t* spl, uint32_t nspl, uint64_t* counts, void* t, size_t* tb, void* s) {
   IO io = io_dev(ki, vi, ko, vo);
   io.counts_out = counts; io.given_spl = spl; io.given_nspl = nspl;
-  if (n && nspl && !spl) return GSS_ERROR_INVALID_VALUE;
+  if (t && n && nspl && !spl) return GSS_ERROR_INVALID_VALUE;
   if (vi) return drive<uint32_t, uint32_t, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
   return drive<uint32_t, NoVal, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
 }
@@ -243,7 +243,28 @@ gss_status gss_partition_by_u64(const uint64_t* ki, const uint64_t* vi, uint64_t
                                 const uint64_t* spl, uint32_t nspl, uint64_t* counts, void* t, size_t* tb, void* s) {
   IO io = io_dev(ki, vi, ko, vo);
   io.counts_out = counts; io.given_spl = spl; io.given_nspl = nspl;
-  if (n && nspl && !spl) return GSS_ERROR_INVALID_VALUE;
+  if (t && n && nspl && !spl) return GSS_ERROR_INVALID_VALUE;
+  if (vi) return drive<uint64_t, uint64_t, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
+  return drive<uint64_t, NoVal, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
+}
+
+gss_status gss_partition_by_eq_u32(const uint32_t* ki, const uint32_t* vi, uint32_t* ko, uint32_t* vo, size_t n,
+                                   const uint32_t* spl, uint32_t nspl, uint64_t* counts, void* t, size_t* tb,
+                                   void* s) {
+  IO io = io_dev(ki, vi, ko, vo);
+  io.counts_out = counts; io.given_spl = spl; io.given_nspl = nspl; io.given_eq = 1;
+  if (t && n && nspl && !spl) return GSS_ERROR_INVALID_VALUE;
+  if (nspl > 127) return GSS_ERROR_INVALID_VALUE;
+  if (vi) return drive<uint32_t, uint32_t, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
+  return drive<uint32_t, NoVal, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
+}
+gss_status gss_partition_by_eq_u64(const uint64_t* ki, const uint64_t* vi, uint64_t* ko, uint64_t* vo, size_t n,
+                                   const uint64_t* spl, uint32_t nspl, uint64_t* counts, void* t, size_t* tb,
+                                   void* s) {
+  IO io = io_dev(ki, vi, ko, vo);
+  io.counts_out = counts; io.given_spl = spl; io.given_nspl = nspl; io.given_eq = 1;
+  if (t && n && nspl && !spl) return GSS_ERROR_INVALID_VALUE;
+  if (nspl > 127) return GSS_ERROR_INVALID_VALUE;
   if (vi) return drive<uint64_t, uint64_t, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
   return drive<uint64_t, NoVal, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
 }

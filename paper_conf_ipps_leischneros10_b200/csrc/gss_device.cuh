@@ -113,6 +113,7 @@ struct Ctx {
   uint32_t* scan_part;
   const Key* given_spl;              // MODE_PARTITION_BY
   uint32_t given_nspl;
+  uint32_t given_eq;                 // MODE_PARTITION_BY in equality mode (ids 2b / 2b+1)
   uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
   uint32_t recompute;                // GSS_FLAG_RECOMPUTE_IDS: no stored ids, Phase 4 re-descends
   uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb;

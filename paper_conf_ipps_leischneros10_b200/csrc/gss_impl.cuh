@@ -460,7 +460,7 @@ struct IO {
   const void* h_kin; const void* h_vin; void* h_kout; void* h_vout;   // host variants
   // partition outputs
   void* spl_out; uint64_t* off_out; uint32_t* info_out; uint64_t* counts_out;
-  const void* given_spl; uint32_t given_nspl;
+  const void* given_spl; uint32_t given_nspl; uint32_t given_eq;
 };
 
 template <class Key, class Val, class Cmp>
@@ -473,6 +473,7 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
     if (io.given_nspl > 1023) return GSS_ERROR_INVALID_VALUE;
     kgiven = 1;
     while (kgiven < io.given_nspl + 1) kgiven <<= 1;
+    if (io.given_eq) kgiven *= 2;                               // K = 2 nspl + 1 counters
   }
   Cfg cfg;
   GSS_TRY(resolve<Key, Val>(up, n, &cfg, kgiven));
@@ -548,6 +549,7 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
       }
       c.given_spl = reinterpret_cast<const Key*>(io.given_spl);
       c.given_nspl = io.given_nspl;
+      c.given_eq = io.given_eq ? 1u : 0u;
     }
     if ((cfg.flags & GSS_FLAG_GRAPH) && mode == MODE_SORT && !host_io && !prof && !(up && up->stats)) {
       // replay (or capture once) the whole launch sequence as a CUDA graph

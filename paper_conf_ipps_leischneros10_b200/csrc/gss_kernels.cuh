@@ -87,7 +87,8 @@ __global__ void k_init(Ctx<Key, Val, IdT> c) {
   B.hist_base = 0; B.spl_base = 0; B.id_base = 0;
   c.bk[0][0] = B;
   LevelCounters& L = c.cnt->lvl[0];
-  L.num_buckets = 1; L.num_tiles = nt; L.hist_alloc = max(kb, 3u) * nt; L.spl_alloc = 2 * kb;
+  const uint32_t kids = (c.mode == MODE_PARTITION_BY && c.given_eq) ? 2 * kb : kb;   // K <= kids - 1
+  L.num_buckets = 1; L.num_tiles = nt; L.hist_alloc = max(kids, 3u) * nt; L.spl_alloc = 2 * kb;
   L.split_elems = c.n;
 }
 
@@ -153,7 +154,10 @@ __global__ void __launch_bounds__(kSampleThreads, 1) k_sample(Ctx<Key, Val, IdT>
 
 // partition_by: the splitters are given (distributed global level).  k_s is
 // the next power of two >= nspl+1; the tree is padded with copies of the
-// largest splitter and ids are clamped to nspl.
+// largest splitter and ids are clamped to nspl.  With given_eq the ids follow
+// the equality rule (R4): 2b for keys strictly between splitters b-1 and b,
+// 2b+1 for keys equal to splitter b (K = 2 nspl + 1), so a run of equal keys
+// lands in one equality bucket whatever the number of equal splitters.
 template <class Key, class Val, class IdT>
 __global__ void k_set_splitters(Ctx<Key, Val, IdT> c) {
   Bucket B = c.bk[0][0];
@@ -169,7 +173,7 @@ __global__ void k_set_splitters(Ctx<Key, Val, IdT> c) {
   }
   if (threadIdx.x == 0) {
     Bucket* g = &c.bk[0][0];
-    g->ks = ks; g->eq = 0; g->K = nspl + 1; g->clamp = 1;
+    g->ks = ks; g->eq = c.given_eq; g->K = c.given_eq ? 2 * nspl + 1 : nspl + 1; g->clamp = 1;
   }
   for (uint32_t i = threadIdx.x; i < B.ntiles; i += blockDim.x) c.tile_bucket[0][B.tile_start + i] = 0;
 }
@@ -232,7 +236,7 @@ __device__ __forceinline__ uint32_t descend_step(uint32_t a, Key e, uint32_t s0,
 // Bucket ids of U keys per lane: the whole descent (plain top levels,
 // bank-replicated middle levels, plain deep levels), then the id rule of the
 // tile's mode (0: range buckets, 1: equality mode R4, 2: clamped ids of
-// partition_by).
+// partition_by, 3: partition_by in equality mode).
 template <int MODE, int U, class Key, class Cmp>
 __device__ __forceinline__ void descend_group(const Key (&e)[U], uint32_t (&id)[U], uint32_t tree_s, uint32_t rep_b,
                                               const Key* spl, uint32_t logk, uint32_t ks, uint32_t K, Cmp less) {
@@ -280,6 +284,11 @@ __device__ __forceinline__ void descend_group(const Key (&e)[U], uint32_t (&id)[
       id[u] = 2 * b + ((b + 1 < ks && !less(e[u], spl[bb])) ? 1u : 0u);
     } else if constexpr (MODE == 2) {
       id[u] = min(b, K - 1);
+    } else if constexpr (MODE == 3) {
+      // given splitters in equality mode (distributed global level): nspl = (K-1)/2
+      // real splitters, the padded tree slots copy the largest; range id 2b, equality id 2b+1
+      const uint32_t nspl = K >> 1, bc = min(b, nspl);
+      id[u] = 2 * bc + ((bc < nspl && !less(e[u], spl[min(bc, nspl - 1)])) ? 1u : 0u);
     } else {
       id[u] = b;
     }
@@ -421,6 +430,8 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
     if (c.recompute) {
       if (B.eq) classify_tile<1, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
       else classify_tile<0, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    } else if (B.eq && B.clamp) {
+      classify_tile<3, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
     } else if (B.eq) {
       classify_tile<1, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
     } else if (B.clamp) {

@@ -293,30 +293,68 @@ def test_recompute_ids_ablation_large(gss, oracle_mod):
         assert int(y[r]) == oracle_mod.select(x, r)
 
 
-def test_distributed_sorter_single_rank_nccl(gss):
-    """The distributed path on one rank over NCCL: sample, sort, partition_by, all-to-all-v, sort."""
+def _dist_world1():
     import torch.distributed as dist
-    from paper_conf_ipps_leischneros10_b200.dist import DistSorter
-    import os
     os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
     os.environ.setdefault("MASTER_PORT", "29561")
-    own = not dist.is_initialized()
-    if own:
+    if not dist.is_initialized():
         dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
-    try:
-        n = 1 << 20
-        x = inputs.keys("gaussian", n, 64, seed=9)
-        v = inputs.values(n, 64)
-        ds = DistSorter("u64", n, True, device="cuda")
-        k, vv, nr = ds(to_dev(x), to_dev(v))
-        assert nr == n
-        np.testing.assert_array_equal(to_host(k), np.sort(x))
-        check_pairs(x, to_host(vv), np.sort(x))
-        assert ds.verify(x)
-        assert ds.count_launches(to_dev(x), to_dev(v)) > 10
-    finally:
-        if own:
-            dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist_name", ["gaussian", "dd", "equal"])
+def test_distributed_sorter_single_rank_nccl(gss, oracle_mod, width, pairs, dist_name):
+    """gss_dist_sort_* on one rank over NCCL: (n, capacity) all-gather, sample all-gather,
+    sample sort, splitters, equality-mode partition, counts all-gather, plan, NCCL
+    send/recv to itself, local sort -- keys equal the oracle's."""
+    from paper_conf_ipps_leischneros10_b200.dist import DistSorter
+    _dist_world1()
+    n = (1 << 20) + 17
+    x = inputs.keys(dist_name, n, width, seed=9)
+    v = inputs.values(n, width) if pairs else None
+    ds = DistSorter(f"u{width}", n, pairs)
+    for _ in range(2):
+        k, vv, nr = ds(to_dev(x), to_dev(v) if pairs else None)
+    assert nr == n
+    ok, _, _ = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=4096))
+    np.testing.assert_array_equal(to_host(k), ok)
+    if pairs:
+        check_pairs(x, to_host(vv), ok)
+    assert ds.verify(x, v)
+    send, recv, cuts = ds.last_exchange()
+    assert send == [n] and recv == [n] and cuts == [0, n]
+
+
+def test_distributed_capacity_error(gss):
+    from paper_conf_ipps_leischneros10_b200.dist import DistSorter
+    _dist_world1()
+    n = 1 << 16
+    x = inputs.keys("uniform", n, 64, seed=2)
+    ds = DistSorter("u64", n, False, capacity=n - 1)
+    with pytest.raises(RuntimeError, match="GSS_ERROR_CAPACITY"):
+        ds(to_dev(x))
+
+
+@pytest.mark.parametrize("width", [32, 64])
+@pytest.mark.parametrize("nspl", [0, 1, 3, 7, 100])
+def test_partition_by_eq_mode(gss, width, nspl):
+    """gss_partition_by_eq: ids 2b / 2b+1 (R4 with given, possibly repeated, splitters),
+    stable partition and counts bit-exact against the plain definition."""
+    n = 5 * 65536 + 1234
+    x = inputs.keys("and3", n, width, seed=nspl + 1)
+    v = inputs.values(n, width)
+    rng = np.random.default_rng(nspl)
+    spl = np.sort(x[rng.integers(0, n, size=nspl)]) if nspl else x[:0]
+    if nspl >= 3:
+        spl[1] = spl[2]                                      # a duplicate splitter
+    ko, vo, cnt = gss.partition_by(to_dev(x), to_dev(v), to_dev(spl), eq=True)
+    b = np.searchsorted(spl, x, side="left")
+    hit = (b < nspl) & (x == spl[np.minimum(b, max(nspl - 1, 0))]) if nspl else np.zeros(n, bool)
+    ids = 2 * b + hit
+    order = np.argsort(ids, kind="stable")
+    np.testing.assert_array_equal(to_host(ko), x[order])
+    np.testing.assert_array_equal(to_host(vo), v[order])
+    np.testing.assert_array_equal(to_host(cnt), np.bincount(ids, minlength=2 * nspl + 1))
 
 
 @pytest.mark.parametrize("width,pairs", KINDS)
