@@ -120,6 +120,9 @@ typedef struct gss_params {
                                       CUDA graph on first use and replay it on later calls
                                       with identical buffers, n and parameters (launch-bound
                                       sizes); ignored with stats or a profiler              */
+#define GSS_FLAG_SCATTER_REGS 32u  /* Phase 4 writes bucket runs with per-key shared loads and
+                                      coalesced global stores (the round-1 scatter; ablation)
+                                      instead of bulk copies (cp.async.bulk) of each run      */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets of two or more warps with one more
                                       sample-sort split inside the SM + warp merge sorts of
                                       packed segments; ablation: on B200 its

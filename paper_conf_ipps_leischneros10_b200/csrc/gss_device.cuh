@@ -499,8 +499,10 @@ struct CtaSort {
       for (int st = w; st > 0; st >>= 1) {
 #endif
         const int pr = j + st - 1;
-        const int pc = min(pr, hi - 1);                     // clamped probe: the loads stay inside the pair
-        const Key b = lds_key(sk, bEnd - (diag - 1 - pc)), a = lds_key(sk, ps + pc);
+        const int pc = min(pr, hi - 1);
+        // clamped probe addresses: the loads stay inside the pair even when its range is empty
+        // (hi == 0), where the result is discarded -- no read of a slot another warp may be storing
+        const Key b = lds_key(sk, max(bEnd - (diag - 1 - pc), ps + aLen)), a = lds_key(sk, max(ps + pc, ps));
         j = (pr < hi) & !less(b, a) ? pr + 1 : j;
       }
       ia = j;
@@ -515,8 +517,9 @@ struct CtaSort {
       for (int st = w; st > 0; st >>= 1) {
 #endif
         const int pr = j + st - 1;
-        const int pc = min(pr, hi - 1);                     // clamped probe (at most one slot past the pair)
-        const Key a = lds_key(sk, ps + diag - 1 - pc), b = lds_key(sk, bEnd - pc);
+        const int pc = min(pr, hi - 1);
+        // clamped probe addresses: inside the pair even when its range is empty (hi == 0, result discarded)
+        const Key a = lds_key(sk, min(ps + diag - 1 - pc, ps + aLen - 1)), b = lds_key(sk, min(bEnd - pc, bEnd));
         j = (pr < hi) & !less(a, b) ? pr + 1 : j;
       }
       ia = diag - j;

@@ -147,7 +147,9 @@ gss_status dist_layout(int P, size_t n_local, size_t cap, const gss_params* p, D
   DTRY(Ops::sort(nullptr, nullptr, PS, nullptr, &tb, nullptr, &sp));
   L->smp_temp = tb;
   tb = 0;
-  DTRY(Ops::part(nullptr, nullptr, nullptr, nullptr, n_local, nullptr, (uint32_t)(P - 1), nullptr, nullptr, &tb, nullptr));
+  // the query must name the instantiation: a non-null value pointer selects the key-value one
+  const Key* vsel = KV ? reinterpret_cast<const Key*>(alignof(Key)) : nullptr;
+  DTRY(Ops::part(nullptr, vsel, nullptr, nullptr, n_local, nullptr, (uint32_t)(P - 1), nullptr, nullptr, &tb, nullptr));
   L->part_temp = tb;
   tb = 0;
   if constexpr (KV) DTRY(Ops::sort_pairs(nullptr, nullptr, nullptr, nullptr, cap, nullptr, &tb, nullptr, &sp));

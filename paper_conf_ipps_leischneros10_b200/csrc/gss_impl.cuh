@@ -347,6 +347,15 @@ struct Engine {
     const size_t sm_sf = ScatterFastSmem<Key, Val, IdT>::bytes(kmax);
     GSS_TRY(set_smem(ksf, sm_sf));
     const int g_sf = grid_for(ksf, kScatterThreads, sm_sf, di.sms);
+    // default sort scatter: bulk-copy stores, two staging buffers when two CTAs still fit an SM
+    using SBS = ScatterBulkSmem<Key, Val, IdT>;
+    const bool bulk2 = SBS::bytes(kmax, 2) <= 113 * 1024;
+    auto ksb = bulk2 ? k_scatter_bulk<Key, Val, IdT, 2> : k_scatter_bulk<Key, Val, IdT, 1>;
+    const size_t sm_sb = SBS::bytes(kmax, bulk2 ? 2 : 1);
+    GSS_TRY(set_smem(ksb, sm_sb));
+    const int g_sb = grid_for(ksb, kScatterThreads, sm_sb, di.sms);
+    const bool use_bulk = !c.stable && !c.recompute &&
+                          !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters | GSS_FLAG_SCATTER_REGS));
     auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
     const size_t sm_sd = (size_t)kmax * 4;
     GSS_TRY(set_smem(ksd, sm_sd));
@@ -365,7 +374,9 @@ struct Engine {
       // default and stable ranks (R7, GSS_FLAG_STABLE): k_scatter with per-warp counters (deterministic);
       // ablations: k_scatter_fast (one counter set per CTA: atomic order across warps is not
       // deterministic) and the paper's direct scatter (k_scatter_direct)
-      if (c.stable || !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters))) {
+      if (use_bulk) {
+        GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksb<<<g_sb, kScatterThreads, sm_sb, s>>>(c, l, kmax); }));
+      } else if (c.stable || !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters))) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));
       } else if (cfg.flags & kFlagScatterCtaCounters) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksf<<<g_sf, kScatterThreads, sm_sf, s>>>(c, l, kmax); }));

@@ -860,6 +860,260 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
   }
 }
 
+// ---------------------------------------------------------------------------
+// Phase 4 with bulk-copy stores (the default sort scatter on B200).  The
+// chunk is ranked and reordered by bucket id in shared memory as in
+// k_scatter, but the bucket runs leave shared memory through the TMA bulk-copy
+// engine (cp.async.bulk.global.shared::cta, SASS UBLKCP) instead of per-key
+// LDS + STG: one thread per bucket id issues its run's 16-byte-aligned middle
+// as one asynchronous copy and stores at most A-1 head and A-1 tail elements
+// itself (A = 16 / key bytes).  Each run's staging slot is placed so that it
+// has the same alignment modulo 16 bytes as its global destination, which
+// costs at most A-1 slots per id.  The copies of chunk c drain while chunk
+// c+1 is ranked (NBUF = 2 staging buffers; 1 where shared memory is short).
+// Per chunk: 5 barriers (the paper's presorting, with the write
+// phase handed to the copy engine).
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ void bulk_s2g(void* gdst, uint32_t ssrc, uint32_t bytes) {
+  asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(gdst), "r"(ssrc), "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void bulk_wait_read() { asm volatile("cp.async.bulk.wait_group.read %0;" ::"n"(N) : "memory"); }
+__device__ __forceinline__ void bulk_wait_all() { asm volatile("cp.async.bulk.wait_group 0;" ::: "memory"); }
+__device__ __forceinline__ void fence_proxy_async_smem() { asm volatile("fence.proxy.async.shared::cta;" ::: "memory"); }
+
+// Exclusive scan of one value per thread with two barriers (no trailing
+// barrier: the caller's next barrier protects s_part).
+template <int NT>
+__device__ __forceinline__ uint32_t block_exclusive_scan2(uint32_t x, uint32_t* s_warp) {
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  uint32_t inc = x;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(kFull, inc, o);
+    if (lane >= o) inc += y;
+  }
+  if (lane == 31) s_warp[w] = inc;
+  __syncthreads();
+  if (w == 0) {
+    const uint32_t v = lane < NT / 32 ? s_warp[lane] : 0;
+    uint32_t vi = v;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(kFull, vi, o);
+      if (lane >= o) vi += y;
+    }
+    if (lane < NT / 32) s_warp[32 + lane] = vi - v;
+  }
+  __syncthreads();
+  return s_warp[32 + w] + inc - x;
+}
+
+template <class Key, class Val, class IdT>
+struct ScatterBulkSmem {
+  static constexpr uint32_t A = 16 / sizeof(Key);            // keys per 16 bytes
+  __host__ __device__ static uint32_t stage_len(uint32_t kmax) {
+    constexpr uint32_t C = (uint32_t)kScatterThreads * (uint32_t)scatter_iter<Key, Val>();
+    return C + kmax * (A - 1) + A;
+  }
+  __host__ __device__ static size_t head_bytes(uint32_t kmax) {
+    return (((size_t)kmax * 3 + (size_t)(kScatterThreads / 32) * kmax) * 4 + 64 * 4 + 15) & ~size_t(15);
+  }
+  __host__ __device__ static size_t key_bytes(uint32_t kmax) { return ((size_t)stage_len(kmax) * sizeof(Key) + 15) & ~size_t(15); }
+  __host__ __device__ static size_t val_bytes(uint32_t kmax) {
+    return kHasVal<Val> ? (((size_t)stage_len(kmax) * sizeof(Val) + 15) & ~size_t(15)) : 0;
+  }
+  static size_t bytes(uint32_t kmax, int nbuf) { return head_bytes(kmax) + (size_t)nbuf * (key_bytes(kmax) + val_bytes(kmax)); }
+};
+
+template <class Key, class Val, class IdT, int NBUF>
+__global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
+    k_scatter_bulk(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  constexpr int kScatterIter = scatter_iter<Key, Val>();
+  constexpr int kChunk = kScatterThreads * kScatterIter;
+  constexpr int NW = kScatterThreads / 32;
+  using SM = ScatterBulkSmem<Key, Val, IdT>;
+  constexpr uint32_t A = SM::A;
+  static_assert(sizeof(Val) == sizeof(Key) || !kHasVal<Val>, "values have the key's width");
+  uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);       // next global index of each id (this tile)
+  uint32_t* rstart = gbase + kmax;                                // staging slot of each id's run (this chunk)
+  uint32_t* rlen = rstart + kmax;                                 // run length of each id (this chunk)
+  uint32_t* wcnt = rlen + kmax;                                   // per-warp counters, then per-warp offsets
+  uint32_t* s_warp = wcnt + NW * kmax;                            // 64 words of scan scratch
+  Key* stage_k = reinterpret_cast<Key*>(smem_raw + SM::head_bytes(kmax));
+  Val* stage_v = reinterpret_cast<Val*>(smem_raw + SM::head_bytes(kmax) + (size_t)NBUF * SM::key_bytes(kmax));
+  const uint32_t SL = SM::stage_len(kmax);
+
+  const uint32_t slot = level & 1;
+  const uint32_t nt = c.cnt->lvl[level].num_tiles;
+  const uint32_t sb = c.src(level), db = c.dst(level);
+  const Key* ksrc = c.keys(sb);
+  Key* kdst = c.wkeys(db);
+  const Val* vsrc = nullptr;
+  Val* vdst = nullptr;
+  if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
+  const IdT* idsrc = c.ids;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  uint32_t* wc = wcnt + w * kmax;
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
+  const uint32_t q0 = w * (32 * kScatterIter) + lane;
+
+  uint32_t t = blockIdx.x;
+  if (t >= nt) return;
+  uint32_t beg, len, K, idb;
+  auto tile_info = [&](uint32_t tt) {
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t tl = tt - B.tile_start;
+    beg = B.lo + tl * c.T;
+    len = min(c.T, B.m - tl * c.T);
+    K = B.K;
+    idb = B.id_base + tl * c.T;
+  };
+  // ids owned by this thread in the scan and the write phase, fixed for the
+  // kernel (gbase, rstart, rlen of an id are only touched by its owner)
+  const uint32_t per = (kmax + kScatterThreads - 1) / kScatterThreads, i0 = threadIdx.x * per;
+  auto load_gbase = [&](uint32_t tt) {                            // owner threads only: no barrier needed
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
+    const uint32_t tl = tt - B.tile_start;
+    const uint32_t* hist = c.hist[slot] + B.hist_base;
+    const uint32_t hb = hist[0];
+    for (uint32_t j = 0; j < per; j++) {
+      const uint32_t id = i0 + j;
+      if (id < B.K) gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
+    }
+  };
+  tile_info(t);
+  load_gbase(t);
+  Key pk[kScatterIter];
+  Val pv[kScatterIter];
+  uint32_t pid[kScatterIter];
+  auto load_chunk = [&](uint32_t cbeg, uint32_t cid, uint32_t clen) {
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      const uint32_t q = q0 + it * 32;
+      pid[it] = 0xffffffffu;
+      if (q < clen) {
+        pk[it] = ksrc[cbeg + q];
+        pid[it] = idsrc[cid + q];
+        if constexpr (kHasVal<Val>) pv[it] = vsrc[cbeg + q];
+      }
+    }
+  };
+  uint32_t c0 = 0, buf = 0;
+  load_chunk(beg, idb, min((uint32_t)kChunk, len));
+  for (;;) {
+    Key kk[kScatterIter];
+    Val vv[kScatterIter];
+    uint32_t iid[kScatterIter];
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      kk[it] = pk[it];
+      iid[it] = pid[it];
+      if constexpr (kHasVal<Val>) vv[it] = pv[it];
+    }
+    const uint32_t cur_K = K;
+    for (uint32_t id = lane; id < cur_K; id += 32) wc[id] = 0;
+    __syncwarp();
+    // ranks within (warp, id): one shared atomic per key on the warp's own counters
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      const uint32_t r = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (iid[it] & 0xffffu), 1u);
+      iid[it] = iid[it] == 0xffffffffu ? iid[it] : (r << 16) | iid[it];
+    }
+    // the staging buffer written below was last read by the copies issued NBUF chunks ago
+    bulk_wait_read<NBUF - 1>();
+    __syncthreads();                                                // B1: counters complete
+    // chunk totals per id, aligned run slots, every warp's start inside each run
+    uint32_t tsum = 0;
+    for (uint32_t j = 0; j < per; j++) {
+      const uint32_t id = i0 + j;
+      if (id < cur_K) {
+        uint32_t tt = 0;
+#pragma unroll
+        for (int q = 0; q < NW; q++) tt += wcnt[q * kmax + id];
+        rlen[id] = tt;
+        tsum += tt + (A - 1);
+      }
+    }
+    uint32_t ex = block_exclusive_scan2<kScatterThreads>(tsum, s_warp);
+    for (uint32_t j = 0; j < per; j++) {
+      const uint32_t id = i0 + j;
+      if (id < cur_K) {
+        const uint32_t L = rlen[id];
+        const uint32_t st = ex + ((gbase[id] - ex) & (A - 1));      // staging slot == global index (mod A)
+        rstart[id] = st;
+        uint32_t run = st;
+#pragma unroll
+        for (int q = 0; q < NW; q++) {
+          const uint32_t x = wcnt[q * kmax + id];
+          wcnt[q * kmax + id] = run;
+          run += x;
+        }
+        ex += L + (A - 1);
+      }
+    }
+    __syncthreads();                                                // B2: run slots known
+    Key* sk = stage_k + (size_t)buf * (SM::key_bytes(kmax) / sizeof(Key));
+    Val* sv = nullptr;
+    if constexpr (kHasVal<Val>) sv = stage_v + (size_t)buf * (SM::val_bytes(kmax) / sizeof(Val));
+#pragma unroll
+    for (int it = 0; it < kScatterIter; it++) {
+      if (iid[it] != 0xffffffffu) {
+        const uint32_t pos = wc[iid[it] & 0xffffu] + (iid[it] >> 16);
+        sk[pos] = kk[it];
+        if constexpr (kHasVal<Val>) sv[pos] = vv[it];
+      }
+    }
+    fence_proxy_async_smem();                                       // generic-proxy stores -> bulk copies
+    __syncthreads();                                                // B3: the chunk is staged
+    // advance and prefetch the next chunk (possibly of the next tile)
+    bool done = false, new_tile = false;
+    c0 += kChunk;
+    if (c0 >= len) {
+      t += gridDim.x;
+      c0 = 0;
+      if (t >= nt) done = true;
+      else { tile_info(t); new_tile = true; }
+    }
+    if (!done) load_chunk(beg + c0, idb + c0, min((uint32_t)kChunk, len - c0));
+    // write this chunk's runs: head / tail elements by the owner, the aligned middle by the copy engine
+    const uint32_t sk_s = (uint32_t)__cvta_generic_to_shared(sk);
+    uint32_t sv_s = 0;
+    if constexpr (kHasVal<Val>) sv_s = (uint32_t)__cvta_generic_to_shared(sv);
+    for (uint32_t j = 0; j < per; j++) {
+      const uint32_t id = i0 + j;
+      if (id >= cur_K) break;
+      const uint32_t L = rlen[id];
+      if (!L) continue;
+      const uint32_t g = gbase[id], st = rstart[id];
+      const uint32_t head = min(L, (A - (g & (A - 1))) & (A - 1));
+      const uint32_t mid_end = head + ((L - head) & ~(A - 1));
+      for (uint32_t h = 0; h < head; h++) {
+        kdst[g + h] = sk[st + h];
+        if constexpr (kHasVal<Val>) vdst[g + h] = sv[st + h];
+      }
+      if (mid_end > head) {
+        bulk_s2g(kdst + g + head, sk_s + (st + head) * (uint32_t)sizeof(Key), (mid_end - head) * (uint32_t)sizeof(Key));
+        if constexpr (kHasVal<Val>)
+          bulk_s2g(vdst + g + head, sv_s + (st + head) * (uint32_t)sizeof(Val), (mid_end - head) * (uint32_t)sizeof(Val));
+      }
+      for (uint32_t h = mid_end; h < L; h++) {
+        kdst[g + h] = sk[st + h];
+        if constexpr (kHasVal<Val>) vdst[g + h] = sv[st + h];
+      }
+      gbase[id] = g + L;
+    }
+    bulk_commit();
+    if constexpr (NBUF == 2) buf ^= 1u;
+    if (done) break;
+    if (new_tile) load_gbase(t);
+  }
+  bulk_wait_all();
+}
+
 // Phase 4, default variant (R7: a partition, not stable).  Every key takes
 // its rank within (chunk, id) from one shared-memory atomic on the CTA's
 // counter for its id; warp 0 scans the K chunk totals into staged run
