@@ -269,6 +269,38 @@ gss_status gss_partition_by_eq_u64(const uint64_t* ki, const uint64_t* vi, uint6
   return drive<uint64_t, NoVal, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
 }
 
+// Internal, not part of gss.h: the two phases of the fused global level of the
+// distributed sort (gss_dist.cu).  Phase 1 = equality-mode classification of
+// keys_in by the splitters, the per-tile histograms and their scan, and the
+// 2*nspl+1 bucket counts; phase 2 (same temp, called after phase 1) = the
+// scatter of that partition straight into the remote segments (peer windows).
+// kbuf/vbuf: any device buffers of n elements disjoint from the inputs (the
+// partition is never written locally).
+}  // extern "C"
+template <class Key>
+static gss_status dist_level(const Key* ki, const Key* vi, Key* kbuf, Key* vbuf, size_t n, const Key* spl,
+                             uint32_t nspl, uint64_t* counts, const void* remote, uint32_t nremote, uint32_t phase,
+                             void* t, size_t* tb, void* s) {
+  IO io = io_dev(ki, vi, kbuf, vbuf);
+  io.counts_out = counts; io.given_spl = spl; io.given_nspl = nspl; io.given_eq = 1;
+  io.unstable = 1; io.phase = phase; io.remote = remote; io.nremote = nremote;
+  if (nspl > 127 || nremote > 64 || phase < 1 || phase > 2) return GSS_ERROR_INVALID_VALUE;
+  if (t && phase == 2 && !remote) return GSS_ERROR_INVALID_VALUE;
+  if (vi) return drive<Key, Key, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
+  return drive<Key, NoVal, Less>(io, n, t, tb, s, nullptr, MODE_PARTITION_BY, false);
+}
+extern "C" {
+gss_status gssi_dist_level_u32(const uint32_t* ki, const uint32_t* vi, uint32_t* kb, uint32_t* vb, size_t n,
+                               const uint32_t* spl, uint32_t nspl, uint64_t* counts, const void* remote,
+                               uint32_t nremote, uint32_t phase, void* t, size_t* tb, void* s) {
+  return dist_level<uint32_t>(ki, vi, kb, vb, n, spl, nspl, counts, remote, nremote, phase, t, tb, s);
+}
+gss_status gssi_dist_level_u64(const uint64_t* ki, const uint64_t* vi, uint64_t* kb, uint64_t* vb, size_t n,
+                               const uint64_t* spl, uint32_t nspl, uint64_t* counts, const void* remote,
+                               uint32_t nremote, uint32_t phase, void* t, size_t* tb, void* s) {
+  return dist_level<uint64_t>(ki, vi, kb, vb, n, spl, nspl, counts, remote, nremote, phase, t, tb, s);
+}
+
 gss_status gss_sample_u32(const uint32_t* keys, size_t n, uint64_t lo_global, uint32_t level_tag, uint64_t seed,
                           uint32_t* out, size_t s, void* stream) {
   if (s == 0) return GSS_SUCCESS;

@@ -78,6 +78,16 @@ struct Bucket {
   uint32_t id_base;        // start of its stored bucket ids (16-byte aligned; tile t at id_base + t*T)
 };
 
+// A destination segment of a partition whose output goes to other GPUs
+// (the fused global level of the distributed sort): partition indices
+// [lo, hi) are stored at kdst[i] / vdst[i] (pointers pre-offset by -lo, into a
+// peer's NCCL symmetric window).
+struct RemoteSeg {
+  uint32_t lo, hi, pad0, pad1;
+  void* kdst;
+  void* vdst;
+};
+
 struct Item {              // a final bucket (small sort / copy / overflow work)
   uint32_t lo, m, buf, pad;
 };
@@ -114,6 +124,8 @@ struct Ctx {
   const Key* given_spl;              // MODE_PARTITION_BY
   uint32_t given_nspl;
   uint32_t given_eq;                 // MODE_PARTITION_BY in equality mode (ids 2b / 2b+1)
+  const RemoteSeg* remote;           // MODE_PARTITION_BY, phase 2: destinations on other GPUs
+  uint32_t nremote;
   uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
   uint32_t recompute;                // GSS_FLAG_RECOMPUTE_IDS: no stored ids, Phase 4 re-descends
   uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb;

@@ -26,8 +26,19 @@
 //     received source-major into keys_out;
 //  7. sort the received range in place (gss_sort).
 // Rank r ends with the r-th contiguous range of the global sorted order.
+//
+// GSS_FLAG_DIST_FUSED fuses steps 4 and 6: the partition is
+// only classified and counted before the plan (gssi_dist_level phase 1); after
+// the plan, its scatter kernel (phase 2, the bulk-copy scatter) stores every
+// bucket run straight into the receiving GPU's NCCL symmetric window
+// (ncclMemAlloc + ncclCommWindowRegister; peer addresses from
+// ncclGetPeerPointer over NVLink), so the exchange overlaps the scatter's HBM
+// traffic and the partitioned shard is never written locally.  A one-element
+// ncclAllReduce then orders every peer's stores before the local sort, which
+// reads the window and writes keys_out.
 #include <cuda_runtime.h>
 #include <nccl.h>
+#include <nccl_device.h>
 
 #include <algorithm>
 #include <cstring>
@@ -35,6 +46,16 @@
 #include <vector>
 
 #include "../../include/gss.h"
+
+extern "C" {
+gss_status gssi_dist_level_u32(const uint32_t* ki, const uint32_t* vi, uint32_t* kb, uint32_t* vb, size_t n,
+                               const uint32_t* spl, uint32_t nspl, uint64_t* counts, const void* remote,
+                               uint32_t nremote, uint32_t phase, void* t, size_t* tb, void* s);
+gss_status gssi_dist_level_u64(const uint64_t* ki, const uint64_t* vi, uint64_t* kb, uint64_t* vb, size_t n,
+                               const uint64_t* spl, uint32_t nspl, uint64_t* counts, const void* remote,
+                               uint32_t nremote, uint32_t phase, void* t, size_t* tb, void* s);
+}
+
 
 namespace {
 
@@ -48,9 +69,22 @@ __global__ void k_pick_splitters(const Key* sorted, uint64_t vs, uint32_t P, Key
   for (uint32_t i = threadIdx.x; i + 1 < P; i += blockDim.x) spl[i] = sorted[((uint64_t)(i + 1) * vs) / P - 1];
 }
 
+// every rank's window base as this GPU addresses it (LSA team over NVLink)
+__global__ void k_peer_ptrs(ncclWindow_t wk, ncclWindow_t wv, int P, void** out) {
+  for (int q = threadIdx.x; q < P; q += blockDim.x) {
+    out[q] = ncclGetPeerPointer(wk, 0, q);
+    out[P + q] = wv ? ncclGetPeerPointer(wv, 0, q) : nullptr;
+  }
+}
+
 template <class Key> struct KeyOps;
 template <> struct KeyOps<uint32_t> {
   static constexpr ncclDataType_t nccl = ncclUint32;
+  static gss_status level(const uint32_t* ki, const uint32_t* vi, uint32_t* kb, uint32_t* vb, size_t n,
+                          const uint32_t* spl, uint32_t nspl, uint64_t* cnt, const void* rem, uint32_t nrem,
+                          uint32_t phase, void* t, size_t* tb, void* s) {
+    return gssi_dist_level_u32(ki, vi, kb, vb, n, spl, nspl, cnt, rem, nrem, phase, t, tb, s);
+  }
   static gss_status sort(const uint32_t* ki, uint32_t* ko, size_t n, void* t, size_t* tb, void* s, const gss_params* p) {
     return gss_sort_u32(ki, ko, n, t, tb, s, p);
   }
@@ -68,6 +102,11 @@ template <> struct KeyOps<uint32_t> {
 };
 template <> struct KeyOps<uint64_t> {
   static constexpr ncclDataType_t nccl = ncclUint64;
+  static gss_status level(const uint64_t* ki, const uint64_t* vi, uint64_t* kb, uint64_t* vb, size_t n,
+                          const uint64_t* spl, uint32_t nspl, uint64_t* cnt, const void* rem, uint32_t nrem,
+                          uint32_t phase, void* t, size_t* tb, void* s) {
+    return gssi_dist_level_u64(ki, vi, kb, vb, n, spl, nspl, cnt, rem, nrem, phase, t, tb, s);
+  }
   static gss_status sort(const uint64_t* ki, uint64_t* ko, size_t n, void* t, size_t* tb, void* s, const gss_params* p) {
     return gss_sort_u64(ki, ko, n, t, tb, s, p);
   }
@@ -103,12 +142,49 @@ template <> struct KeyOps<uint64_t> {
 struct gss_dist {
   ncclComm_t comm = nullptr;
   int rank = 0, P = 1, dev = 0;
-  uint64_t* h_buf = nullptr;       // pinned staging of the two small exchanges
+  uint64_t* h_buf = nullptr;       // pinned staging of the small exchanges and the segment table
   size_t h_cap = 0;
   std::vector<uint64_t> send_cnt, recv_cnt, cuts;   // the last call's exchange plan
+  // fused exchange: symmetric receive windows (keys, values) of wcap elements
+  void* wk = nullptr;
+  void* wv = nullptr;
+  ncclWindow_t win_k = nullptr, win_v = nullptr;
+  size_t wcap = 0, welem = 0;
+  std::vector<void*> peer_k, peer_v;                  // every rank's window, as seen from this GPU
 };
 
 namespace {
+
+// Symmetric receive windows of at least cap elements of w bytes (keys, and values when kv), registered
+// collectively (every rank calls with the same cap), and every rank's window address as seen here.
+gss_status ensure_windows(gss_dist* d, size_t cap, size_t w, bool kv, void** d_ptrs, cudaStream_t s) {
+  if (d->wk && d->wcap >= cap && d->welem == w && (!kv || d->wv)) return GSS_SUCCESS;
+  CTRY(cudaStreamSynchronize(s));
+  if (d->win_k) ncclCommWindowDeregister(d->comm, d->win_k);
+  if (d->win_v) ncclCommWindowDeregister(d->comm, d->win_v);
+  if (d->wk) ncclMemFree(d->wk);
+  if (d->wv) ncclMemFree(d->wv);
+  d->wk = d->wv = nullptr;
+  d->win_k = d->win_v = nullptr;
+  d->wcap = 0;
+  const size_t bytes = align_up(std::max<size_t>(cap, 1) * w, (size_t)1 << 21);
+  NTRY(ncclMemAlloc(&d->wk, bytes));
+  NTRY(ncclCommWindowRegister(d->comm, d->wk, bytes, &d->win_k, NCCL_WIN_COLL_SYMMETRIC));
+  if (kv) {
+    NTRY(ncclMemAlloc(&d->wv, bytes));
+    NTRY(ncclCommWindowRegister(d->comm, d->wv, bytes, &d->win_v, NCCL_WIN_COLL_SYMMETRIC));
+  }
+  k_peer_ptrs<<<1, 64, 0, s>>>(d->win_k, d->win_v, d->P, d_ptrs);
+  CTRY(cudaGetLastError());
+  std::vector<void*> h(2 * (size_t)d->P);
+  CTRY(cudaMemcpyAsync(h.data(), d_ptrs, h.size() * sizeof(void*), cudaMemcpyDeviceToHost, s));
+  CTRY(cudaStreamSynchronize(s));
+  d->peer_k.assign(h.begin(), h.begin() + d->P);
+  d->peer_v.assign(h.begin() + d->P, h.end());
+  d->wcap = bytes / w;
+  d->welem = w;
+  return GSS_SUCCESS;
+}
 
 gss_status host_buf(gss_dist* d, size_t words) {
   if (d->h_cap >= words) return GSS_SUCCESS;
@@ -123,9 +199,11 @@ gss_status host_buf(gss_dist* d, size_t words) {
 template <class Key, class Val>
 struct DistLayout {
   size_t off_meta, off_meta_all, off_smp, off_smp_all, off_smp_sorted, off_smp_temp, off_spl, off_cnt, off_cnt_all,
-      off_part_k, off_part_v, off_part_temp, off_sort_temp, total;
+      off_part_k, off_part_v, off_part_temp, off_sort_temp, off_peer, off_seg, off_one, total;
   size_t smp_temp, part_temp, sort_temp;
 };
+
+inline bool fused_mode(const gss_params* p) { return p && (p->flags & GSS_FLAG_DIST_FUSED); }
 
 // Host view of the internal sub-calls' parameters: the caller's method
 // parameters, without statistics (only the local sort reports them).
@@ -149,7 +227,12 @@ gss_status dist_layout(int P, size_t n_local, size_t cap, const gss_params* p, D
   tb = 0;
   // the query must name the instantiation: a non-null value pointer selects the key-value one
   const Key* vsel = KV ? reinterpret_cast<const Key*>(alignof(Key)) : nullptr;
-  DTRY(Ops::part(nullptr, vsel, nullptr, nullptr, n_local, nullptr, (uint32_t)(P - 1), nullptr, nullptr, &tb, nullptr));
+  const bool fused = fused_mode(p);
+  if (fused)
+    DTRY(Ops::level(nullptr, vsel, nullptr, nullptr, n_local, nullptr, (uint32_t)(P - 1), nullptr, nullptr, 0, 1,
+                    nullptr, &tb, nullptr));
+  else
+    DTRY(Ops::part(nullptr, vsel, nullptr, nullptr, n_local, nullptr, (uint32_t)(P - 1), nullptr, nullptr, &tb, nullptr));
   L->part_temp = tb;
   tb = 0;
   if constexpr (KV) DTRY(Ops::sort_pairs(nullptr, nullptr, nullptr, nullptr, cap, nullptr, &tb, nullptr, &sp));
@@ -167,10 +250,13 @@ gss_status dist_layout(int P, size_t n_local, size_t cap, const gss_params* p, D
   L->off_spl = take((size_t)P * sizeof(Key));
   L->off_cnt = take(K * sizeof(uint64_t));
   L->off_cnt_all = take(K * P * sizeof(uint64_t));
-  L->off_part_k = take(n_local * sizeof(Key));
-  L->off_part_v = KV ? take(n_local * sizeof(Key)) : 0;
+  L->off_part_k = fused ? 0 : take(n_local * sizeof(Key));      // the fused path never writes the partition locally
+  L->off_part_v = (KV && !fused) ? take(n_local * sizeof(Key)) : 0;
   L->off_part_temp = take(L->part_temp);
   L->off_sort_temp = take(L->sort_temp);
+  L->off_peer = take(2 * (size_t)P * sizeof(void*));
+  L->off_seg = take((size_t)P * 32);
+  L->off_one = take(sizeof(uint64_t));
   L->total = o;
   return GSS_SUCCESS;
 }
@@ -196,7 +282,8 @@ gss_status dist_sort(gss_dist* d, const Key* kin, const Key* vin, size_t n_local
   const ncclDataType_t dt = Ops::nccl;
   const uint32_t S = kDistSamples;
   const size_t K = 2 * (size_t)P - 1;
-  DTRY(host_buf(d, std::max<size_t>(2 * (size_t)P, K * P)));
+  DTRY(host_buf(d, std::max<size_t>(2 * (size_t)P, K * P) + 4 * (size_t)P));
+  const bool fused = fused_mode(p);
   uint64_t* h = d->h_buf;
   gss_params sp = sub_params(p, false);
   const uint64_t seed = (p && p->seed) ? p->seed : 5489;
@@ -220,6 +307,11 @@ gss_status dist_sort(gss_dist* d, const Key* kin, const Key* vin, size_t n_local
   }
   d->send_cnt.assign(P, 0); d->recv_cnt.assign(P, 0); d->cuts.assign(P + 1, 0);
   if (N == 0) { *n_out = 0; return GSS_SUCCESS; }
+  if (fused) {
+    // windows sized for the largest capacity of any rank (same call on every rank)
+    const uint64_t maxcap = *std::max_element(caps.begin(), caps.end());
+    DTRY(ensure_windows(d, std::max<uint64_t>(maxcap, 1), sizeof(Key), KV, reinterpret_cast<void**>(at(L.off_peer)), s));
+  }
 
   // 2-3. global sample, identical sorted sample and splitters on every rank
   Key* smp = reinterpret_cast<Key*>(at(L.off_smp));
@@ -251,7 +343,14 @@ gss_status dist_sort(gss_dist* d, const Key* kin, const Key* vin, size_t n_local
   Key* pv = KV ? reinterpret_cast<Key*>(at(L.off_part_v)) : nullptr;
   uint64_t* d_cnt = reinterpret_cast<uint64_t*>(at(L.off_cnt));
   uint64_t* d_cnt_all = reinterpret_cast<uint64_t*>(at(L.off_cnt_all));
-  if (n_local) {
+  Key* wk = reinterpret_cast<Key*>(d->wk);
+  Key* wv = reinterpret_cast<Key*>(d->wv);
+  if (n_local && fused) {
+    // phase 1: classify + counts only (the window is a stand-in output buffer, never written here)
+    tb = L.part_temp;
+    DTRY(Ops::level(kin, KV ? vin : nullptr, wk, KV ? wv : nullptr, n_local, spl, (uint32_t)(P - 1), d_cnt, nullptr, 0,
+                    1, at(L.off_part_temp), &tb, s));
+  } else if (n_local) {
     tb = L.part_temp;
     DTRY(Ops::part(kin, KV ? vin : nullptr, pk, pv, n_local, spl, (uint32_t)(P - 1), d_cnt, at(L.off_part_temp), &tb, s));
   } else {
@@ -266,10 +365,14 @@ gss_status dist_sort(gss_dist* d, const Key* kin, const Key* vin, size_t n_local
   // capacity: every rank checks every rank, so all of them stop together
   bool over = false;
   uint64_t need_me = 0;
+  std::vector<uint64_t> my_off_in(P, 0);                 // where this rank's data starts in rank q's receive layout
   for (int q = 0; q < P; q++) {
     DTRY(gss_dist_plan((uint32_t)P, (uint32_t)q, (uint32_t)K, h, cuts.data(), soff.data(), scnt.data(), rcnt.data()));
     uint64_t need = 0;
-    for (int x = 0; x < P; x++) need += rcnt[x];
+    for (int x = 0; x < P; x++) {
+      if (x == r) my_off_in[q] = need;
+      need += rcnt[x];
+    }
     if (need > caps[q]) over = true;
     if (q == r) need_me = need;
   }
@@ -277,6 +380,39 @@ gss_status dist_sort(gss_dist* d, const Key* kin, const Key* vin, size_t n_local
   d->send_cnt = scnt; d->recv_cnt = rcnt; d->cuts = cuts;
   *n_out = need_me;
   if (over) return GSS_ERROR_CAPACITY;
+
+  if (fused) {
+    // 6'. phase 2: the scatter writes each run into the window of the rank that owns it, at
+    //     (this rank's start in that rank's receive layout) + (partition index - segment start)
+    uint64_t* hs = h + std::max<size_t>(2 * (size_t)P, K * P);
+    for (int q = 0; q < P; q++) {
+      uint32_t* seg = reinterpret_cast<uint32_t*>(hs + 4 * (size_t)q);
+      seg[0] = (uint32_t)soff[q];
+      seg[1] = (uint32_t)(soff[q] + scnt[q]);
+      seg[2] = seg[3] = 0;
+      const int64_t shift = (int64_t)my_off_in[q] - (int64_t)soff[q];
+      Key* kd = reinterpret_cast<Key*>(d->peer_k[q]) + shift;
+      Key* vd = KV ? reinterpret_cast<Key*>(d->peer_v[q]) + shift : nullptr;
+      memcpy(hs + 4 * (size_t)q + 2, &kd, sizeof(void*));
+      memcpy(hs + 4 * (size_t)q + 3, &vd, sizeof(void*));
+    }
+    void* d_seg = at(L.off_seg);
+    CTRY(cudaMemcpyAsync(d_seg, hs, 32 * (size_t)P, cudaMemcpyHostToDevice, s));
+    if (n_local) {
+      tb = L.part_temp;
+      DTRY(Ops::level(kin, KV ? vin : nullptr, wk, KV ? wv : nullptr, n_local, spl, (uint32_t)(P - 1), d_cnt, d_seg,
+                      (uint32_t)P, 2, at(L.off_part_temp), &tb, s));
+    }
+    // every rank's stores into every window are complete before anyone reads its window
+    uint64_t* d_one = reinterpret_cast<uint64_t*>(at(L.off_one));
+    NTRY(ncclAllReduce(d_one, d_one, 1, ncclUint64, ncclSum, d->comm, s));
+    // 7'. local sort: window -> keys_out
+    gss_params lp = sub_params(p, true);
+    tb = L.sort_temp;
+    if constexpr (KV) DTRY(Ops::sort_pairs(wk, wv, kout, vout, need_me, at(L.off_sort_temp), &tb, s, &lp));
+    else DTRY(Ops::sort(wk, kout, need_me, at(L.off_sort_temp), &tb, s, &lp));
+    return GSS_SUCCESS;
+  }
 
   // 6. all-to-all-v over NCCL: one message per peer and array, received source-major
   std::vector<uint64_t> roff(P);
@@ -379,6 +515,11 @@ gss_status gss_dist_create(gss_dist** out, const uint8_t id[128], int rank, int 
 gss_status gss_dist_destroy(gss_dist* d) {
   if (!d) return GSS_ERROR_INVALID_VALUE;
   gss_status st = GSS_SUCCESS;
+  cudaSetDevice(d->dev);
+  if (d->win_k) ncclCommWindowDeregister(d->comm, d->win_k);
+  if (d->win_v) ncclCommWindowDeregister(d->comm, d->win_v);
+  if (d->wk) ncclMemFree(d->wk);
+  if (d->wv) ncclMemFree(d->wv);
   if (d->comm && ncclCommDestroy(d->comm) != ncclSuccess) st = GSS_ERROR_NCCL;
   if (d->h_buf) cudaFreeHost(d->h_buf);
   delete d;

@@ -36,6 +36,7 @@ namespace gssh {
 
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
+inline constexpr uint32_t kFlagScatterBulk = 1u << 29;          // ablation: bulk-copy scatter for 4-byte keys too
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -323,13 +324,14 @@ struct Engine {
 
   // The whole launch sequence.  mode: sort / partition / partition_by.
   static gss_status run(C& c, const Cfg& cfg, int mode, const DeviceInfo& di, cudaStream_t s, gss_profiler* prof,
-                        uint32_t* count) {
-    GSS_TRY(launch(prof, GSS_K_INIT, s, count, [&] { k_init<Key, Val, IdT><<<1, 256, 0, s>>>(c); }));
+                        uint32_t* count, uint32_t phase = 0) {
+    if (phase != 2)
+      GSS_TRY(launch(prof, GSS_K_INIT, s, count, [&] { k_init<Key, Val, IdT><<<1, 256, 0, s>>>(c); }));
     const uint32_t kmax = cfg.kmax;
     // kernels and their shared-memory sizes
     auto ks = k_sample<Key, Val, IdT, Cmp>;
     const size_t sm_sample = CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
-    auto kc = k_classify<Key, Val, IdT, Cmp>;
+    auto kc = mode == MODE_PARTITION_BY ? k_classify<Key, Val, IdT, Cmp, true> : k_classify<Key, Val, IdT, Cmp, false>;
     const size_t sm_cls = cls_smem_bytes<Key>(kmax);
     auto ksc = c.stable ? k_scatter<Key, Val, IdT, Cmp, true>
                         : (c.recompute ? k_scatter<Key, Val, IdT, Cmp, false, true> : k_scatter<Key, Val, IdT, Cmp, false>);
@@ -354,13 +356,17 @@ struct Engine {
     const size_t sm_sb = SBS::bytes(kmax, bulk2 ? 2 : 1);
     GSS_TRY(set_smem(ksb, sm_sb));
     const int g_sb = grid_for(ksb, kScatterThreads, sm_sb, di.sms);
-    const bool use_bulk = !c.stable && !c.recompute &&
-                          !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters | GSS_FLAG_SCATTER_REGS));
+    // bulk copies pay for 8-byte keys (2^28 u64: 2.90 vs 3.11 ms for the two levels; u64 pairs equal);
+    // for 4-byte keys the per-run copies (one warp-serialised UBLKCP each) cost more than the
+    // coalesced per-key stores they replace (2^27 u32: 1.26 vs 1.05 ms), so those keep GSS_FLAG_SCATTER_REGS
+    const bool use_bulk = c.nremote || (!c.stable && !c.recompute && (sizeof(Key) == 8 || (cfg.flags & kFlagScatterBulk)) &&
+                          !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters | GSS_FLAG_SCATTER_REGS)));
     auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
     const size_t sm_sd = (size_t)kmax * 4;
     GSS_TRY(set_smem(ksd, sm_sd));
     const int g_sd = grid_for(ksd, kDirectThreads, sm_sd, di.sms);
     for (uint32_t l = 0; l < c.L; l++) {
+      if (phase != 2) {
       if (mode == MODE_PARTITION_BY) {
         GSS_TRY(launch(prof, GSS_K_SAMPLE, s, count, [&] { k_set_splitters<Key, Val, IdT><<<1, 256, 0, s>>>(c); }));
       } else {
@@ -371,6 +377,8 @@ struct Engine {
                      [&] { k_scan_reduce<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
       GSS_TRY(launch(prof, GSS_K_SCAN, s, count,
                      [&] { k_scan_final<Key, Val, IdT><<<kScanCtas, kScanThreads, 0, s>>>(c, l); }));
+      }
+      if (phase == 1) continue;                                   // the scatter follows in phase 2
       // default and stable ranks (R7, GSS_FLAG_STABLE): k_scatter with per-warp counters (deterministic);
       // ablations: k_scatter_fast (one counter set per CTA: atomic order across warps is not
       // deterministic) and the paper's direct scatter (k_scatter_direct)
@@ -472,6 +480,10 @@ struct IO {
   // partition outputs
   void* spl_out; uint64_t* off_out; uint32_t* info_out; uint64_t* counts_out;
   const void* given_spl; uint32_t given_nspl; uint32_t given_eq;
+  // distributed global level (internal): phase 1 = classify + counts, phase 2 = the scatter
+  // of the same temp state to remote segments; unstable = non-stable (bulk) scatter
+  uint32_t phase, unstable, nremote;
+  const void* remote;
 };
 
 template <class Key, class Val, class Cmp>
@@ -561,6 +573,9 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
       c.given_spl = reinterpret_cast<const Key*>(io.given_spl);
       c.given_nspl = io.given_nspl;
       c.given_eq = io.given_eq ? 1u : 0u;
+      if (io.unstable) c.stable = 0;
+      c.remote = reinterpret_cast<const RemoteSeg*>(io.remote);
+      c.nremote = io.nremote;
     }
     if ((cfg.flags & GSS_FLAG_GRAPH) && mode == MODE_SORT && !host_io && !prof && !(up && up->stats)) {
       // replay (or capture once) the whole launch sequence as a CUDA graph
@@ -601,8 +616,8 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
       if (cudaGraphLaunch(exec, s) != cudaSuccess) { cudaGetLastError(); return GSS_ERROR_CUDA; }
       return GSS_SUCCESS;
     }
-    GSS_TRY(Eng::run(c, cfg, mode, di, s, prof, &count));
-    if (mode != MODE_SORT) {
+    GSS_TRY(Eng::run(c, cfg, mode, di, s, prof, &count, io.phase));
+    if (mode != MODE_SORT && io.phase != 2) {
       GSS_TRY(launch(prof, GSS_K_OTHER, s, &count, [&] {
         k_partition_out<Key, Val, IdT><<<1, 256, 0, s>>>(c, reinterpret_cast<Key*>(io.spl_out), io.off_out,
                                                           io.info_out, io.counts_out);

@@ -374,7 +374,9 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
 // Persistent: CTA b classifies the contiguous tile range [b*per, (b+1)*per),
 // so consecutive tiles mostly share a bucket and its tree stays in shared
 // memory.
-template <class Key, class Val, class IdT, class Cmp>
+// PART: the partition_by modes (2, 3) only; else the sort modes (0, 1): each
+// instantiation holds only the descents it runs (their registers add up).
+template <class Key, class Val, class IdT, class Cmp, bool PART = false>
 #ifndef GSS_CLS_MINB
 #define GSS_CLS_MINB 2
 #endif
@@ -427,15 +429,14 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
     const uint32_t len = min(c.T, B.m - tl * c.T);
     const uint32_t logk = ilog2(B.ks);
     IdT* tids = c.ids + B.id_base + tl * c.T;                  // 16-byte aligned per tile
-    if (c.recompute) {
+    if constexpr (PART) {
+      if (B.eq) classify_tile<3, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+      else classify_tile<2, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+    } else if (c.recompute) {
       if (B.eq) classify_tile<1, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
       else classify_tile<0, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
-    } else if (B.eq && B.clamp) {
-      classify_tile<3, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
     } else if (B.eq) {
       classify_tile<1, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
-    } else if (B.clamp) {
-      classify_tile<2, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
     } else {
       classify_tile<0, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
     }
@@ -911,6 +912,13 @@ __device__ __forceinline__ uint32_t block_exclusive_scan2(uint32_t x, uint32_t* 
   return s_warp[32 + w] + inc - x;
 }
 
+// The segment holding partition index i (segments are sorted and cover the partition).
+__device__ __forceinline__ const RemoteSeg* find_seg(const RemoteSeg* seg, uint32_t nseg, uint32_t i) {
+  uint32_t q = 0;
+  while (q + 1 < nseg && i >= seg[q].hi) q++;
+  return seg + q;
+}
+
 template <class Key, class Val, class IdT>
 struct ScatterBulkSmem {
   static constexpr uint32_t A = 16 / sizeof(Key);            // keys per 16 bytes
@@ -1043,7 +1051,12 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       const uint32_t id = i0 + j;
       if (id < cur_K) {
         const uint32_t L = rlen[id];
-        const uint32_t st = ex + ((gbase[id] - ex) & (A - 1));      // staging slot == global index (mod A)
+        uint32_t dal = gbase[id];                                   // destination element index (mod A)
+        if (c.nremote) {
+          const RemoteSeg* sg = find_seg(c.remote, c.nremote, dal);
+          dal = (uint32_t)(reinterpret_cast<uintptr_t>(reinterpret_cast<Key*>(sg->kdst) + dal) / sizeof(Key));
+        }
+        const uint32_t st = ex + ((dal - ex) & (A - 1));            // staging slot == destination (mod A)
         rstart[id] = st;
         uint32_t run = st;
 #pragma unroll
@@ -1083,26 +1096,45 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     const uint32_t sk_s = (uint32_t)__cvta_generic_to_shared(sk);
     uint32_t sv_s = 0;
     if constexpr (kHasVal<Val>) sv_s = (uint32_t)__cvta_generic_to_shared(sv);
+    // one piece: dst[0..cnt) <- staging[so..so+cnt): head / tail elements by
+    // this thread, the 16-byte-aligned middle by one bulk copy
+    auto put = [&](Key* dk, Val* dv, uint32_t so, uint32_t cnt) {
+      const uint32_t mis = (uint32_t)(reinterpret_cast<uintptr_t>(dk) & 15u) / (uint32_t)sizeof(Key);
+      uint32_t head = min(cnt, (A - mis) & (A - 1));
+      // the staging slot matches the destination modulo 16 bytes (else: element by element)
+      if (((sk_s + (so + head) * (uint32_t)sizeof(Key)) & 15u) != 0) head = cnt;
+      const uint32_t mid_end = head + ((cnt - head) & ~(A - 1));
+      for (uint32_t h = 0; h < head; h++) {
+        dk[h] = sk[so + h];
+        if constexpr (kHasVal<Val>) dv[h] = sv[so + h];
+      }
+      if (mid_end > head) {
+        bulk_s2g(dk + head, sk_s + (so + head) * (uint32_t)sizeof(Key), (mid_end - head) * (uint32_t)sizeof(Key));
+        if constexpr (kHasVal<Val>)
+          bulk_s2g(dv + head, sv_s + (so + head) * (uint32_t)sizeof(Val), (mid_end - head) * (uint32_t)sizeof(Val));
+      }
+      for (uint32_t h = mid_end; h < cnt; h++) {
+        dk[h] = sk[so + h];
+        if constexpr (kHasVal<Val>) dv[h] = sv[so + h];
+      }
+    };
     for (uint32_t j = 0; j < per; j++) {
       const uint32_t id = i0 + j;
       if (id >= cur_K) break;
       const uint32_t L = rlen[id];
       if (!L) continue;
       const uint32_t g = gbase[id], st = rstart[id];
-      const uint32_t head = min(L, (A - (g & (A - 1))) & (A - 1));
-      const uint32_t mid_end = head + ((L - head) & ~(A - 1));
-      for (uint32_t h = 0; h < head; h++) {
-        kdst[g + h] = sk[st + h];
-        if constexpr (kHasVal<Val>) vdst[g + h] = sv[st + h];
-      }
-      if (mid_end > head) {
-        bulk_s2g(kdst + g + head, sk_s + (st + head) * (uint32_t)sizeof(Key), (mid_end - head) * (uint32_t)sizeof(Key));
-        if constexpr (kHasVal<Val>)
-          bulk_s2g(vdst + g + head, sv_s + (st + head) * (uint32_t)sizeof(Val), (mid_end - head) * (uint32_t)sizeof(Val));
-      }
-      for (uint32_t h = mid_end; h < L; h++) {
-        kdst[g + h] = sk[st + h];
-        if constexpr (kHasVal<Val>) vdst[g + h] = sv[st + h];
+      if (!c.nremote) {
+        put(kdst + g, kHasVal<Val> ? vdst + g : nullptr, st, L);
+      } else {
+        // fused exchange: the run goes to the GPUs owning its partition indices
+        for (uint32_t done = 0; done < L;) {
+          const RemoteSeg* sg = find_seg(c.remote, c.nremote, g + done);
+          const uint32_t cnt = min(L - done, sg->hi - (g + done));
+          put(reinterpret_cast<Key*>(sg->kdst) + g + done,
+              kHasVal<Val> ? reinterpret_cast<Val*>(sg->vdst) + g + done : nullptr, st + done, cnt);
+          done += cnt;
+        }
       }
       gbase[id] = g + L;
     }
@@ -1112,6 +1144,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     if (new_tile) load_gbase(t);
   }
   bulk_wait_all();
+  if (c.nremote) __threadfence_system();                          // peer stores visible before the exchange barrier
 }
 
 // Phase 4, default variant (R7: a partition, not stable).  Every key takes

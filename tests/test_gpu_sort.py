@@ -303,16 +303,18 @@ def _dist_world1():
 
 @pytest.mark.parametrize("width,pairs", KINDS)
 @pytest.mark.parametrize("dist_name", ["gaussian", "dd", "equal"])
-def test_distributed_sorter_single_rank_nccl(gss, oracle_mod, width, pairs, dist_name):
+@pytest.mark.parametrize("fused", [False, True])
+def test_distributed_sorter_single_rank_nccl(gss, oracle_mod, width, pairs, dist_name, fused):
     """gss_dist_sort_* on one rank over NCCL: (n, capacity) all-gather, sample all-gather,
     sample sort, splitters, equality-mode partition, counts all-gather, plan, NCCL
-    send/recv to itself, local sort -- keys equal the oracle's."""
+    send/recv to itself (or, fused = GSS_FLAG_DIST_FUSED, the scatter writing into the
+    rank's NCCL symmetric window), local sort -- keys equal the oracle's."""
     from paper_conf_ipps_leischneros10_b200.dist import DistSorter
     _dist_world1()
     n = (1 << 20) + 17
     x = inputs.keys(dist_name, n, width, seed=9)
     v = inputs.values(n, width) if pairs else None
-    ds = DistSorter(f"u{width}", n, pairs)
+    ds = DistSorter(f"u{width}", n, pairs, flags=64 if fused else 0)
     for _ in range(2):
         k, vv, nr = ds(to_dev(x), to_dev(v) if pairs else None)
     assert nr == n
