@@ -443,6 +443,8 @@ def run_dist(args, wl):
     kind = f"u{bits}"
     params = workload_params(wl)
     params.pop("flags", None)                  # no graph replay: the received count varies per call
+    if args.fused:
+        params["flags"] = 64                   # GSS_FLAG_DIST_FUSED
     x = inputs.keys(distname, n * world, bits, seed=1, start=rank * n, count=n)
     hv = inputs.values(n, bits, start=rank * n) if pairs else None
     dkeys = torch.from_numpy(x).to(dev)
@@ -587,6 +589,8 @@ def main():
     ap.add_argument("--workload", default=DEFAULT_WORKLOAD, choices=sorted(WORKLOADS))
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--force-dist", action="store_true", help="use the distributed path even on one GPU")
+    ap.add_argument("--fused", action="store_true", help="distributed path: fused scatter into peer windows "
+                                                         "(GSS_FLAG_DIST_FUSED)")
     args = ap.parse_args()
     if args.warmup < 3 and args.impl == "ours":
         args.warmup = 3

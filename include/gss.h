@@ -159,11 +159,24 @@ gss_status gss_sort_pairs_u64(const uint64_t* keys_in, const uint64_t* vals_in,
                               uint64_t* keys_out, uint64_t* vals_out, size_t n,
                               void* temp, size_t* temp_bytes, void* stream, const gss_params* p);
 
-/* Descending order: the same kernels instantiated with less(a,b) = a > b,
- * exercising the comparator-only contract. */
+/* Descending order (every integer kind): the same kernels instantiated with
+ * less(a,b) = a > b, exercising the comparator-only contract. */
 gss_status gss_sort_u64_descending(const uint64_t* keys_in, uint64_t* keys_out, size_t n,
                                    void* temp, size_t* temp_bytes, void* stream,
                                    const gss_params* p);
+gss_status gss_sort_u32_descending(const uint32_t* keys_in, uint32_t* keys_out, size_t n,
+                                   void* temp, size_t* temp_bytes, void* stream,
+                                   const gss_params* p);
+gss_status gss_sort_pairs_u32_descending(const uint32_t* keys_in, const uint32_t* vals_in,
+                                         uint32_t* keys_out, uint32_t* vals_out, size_t n,
+                                         void* temp, size_t* temp_bytes, void* stream,
+                                         const gss_params* p);
+gss_status gss_sort_pairs_u64_descending(const uint64_t* keys_in, const uint64_t* vals_in,
+                                         uint64_t* keys_out, uint64_t* vals_out, size_t n,
+                                         void* temp, size_t* temp_bytes, void* stream,
+                                         const gss_params* p);
+/* Any other key type or strict weak order: include/gss.hpp (gss::sort<Key, Less>,
+ * gss::sort_pairs<Key, Val, Less>), compiled into the caller's own nvcc translation unit. */
 
 /* Floating-point keys under the IEEE-754 total order (-NaN < -inf < ... < -0 <
  * +0 < ... < +inf < +NaN): the same kernels with a different comparator

@@ -85,13 +85,13 @@ def _lib():
         lib = ctypes.CDLL(_build.LIB)
         P = ctypes.POINTER(_Params)
         szp = ctypes.POINTER(_sz)
-        for name in ("gss_sort_u32", "gss_sort_u64", "gss_sort_u64_descending", "gss_sort_f32", "gss_sort_f64",
-                     "gss_sort_host_u32", "gss_sort_host_u64"):
+        for name in ("gss_sort_u32", "gss_sort_u64", "gss_sort_u64_descending", "gss_sort_u32_descending",
+                     "gss_sort_f32", "gss_sort_f64", "gss_sort_host_u32", "gss_sort_host_u64"):
             f = getattr(lib, name)
             f.restype = ctypes.c_int
             f.argtypes = [_vp, _vp, _sz, _vp, szp, _vp, P]
         for name in ("gss_sort_pairs_u32", "gss_sort_pairs_u64", "gss_sort_host_pairs_u32",
-                     "gss_sort_host_pairs_u64"):
+                     "gss_sort_host_pairs_u64", "gss_sort_pairs_u32_descending", "gss_sort_pairs_u64_descending"):
             f = getattr(lib, name)
             f.restype = ctypes.c_int
             f.argtypes = [_vp, _vp, _vp, _vp, _sz, _vp, szp, _vp, P]
@@ -253,21 +253,19 @@ def _sort(lib, keys, values, out, values_out, descending, stats, profiler, strea
     if values is not None:
         if kind in ("f32", "f64"):
             raise NotImplementedError("float keys are exported keys-only")
-        if descending:
-            raise NotImplementedError("descending order is exported for keys-only u64")
         values = values.contiguous()
         if values.dtype != keys.dtype or values.numel() != n or values.device != keys.device:
             raise TypeError("values must have the key dtype, length and device")
         _check_out(values_out, values, "values_out")
         vout = torch.empty_like(values) if values_out is None else values_out
-        fn = getattr(lib, f"gss_sort_pairs_{kind}")
+        fn = getattr(lib, f"gss_sort_pairs_{kind}{'_descending' if descending else ''}")
         head = (_ptr(keys), _ptr(values), _ptr(out), _ptr(vout), n)
     else:
         vout = None
         if descending:
-            if kind != "u64":
-                raise NotImplementedError("descending order is exported for keys-only u64")
-            fn = lib.gss_sort_u64_descending
+            if kind not in ("u32", "u64"):
+                raise NotImplementedError("descending order is exported for u32 / u64 keys")
+            fn = getattr(lib, f"gss_sort_{kind}_descending")
         else:
             fn = getattr(lib, f"gss_sort_{kind}")
         head = (_ptr(keys), _ptr(out), n)
@@ -305,9 +303,9 @@ class Sorter:
         self.params = params
         self.temp = torch.empty(max(temp_bytes(kind, n, pairs, **params), 1), dtype=torch.uint8, device=self.device)
         if descending:
-            if pairs or kind != "u64":
-                raise NotImplementedError("descending order is exported for keys-only u64")
-            self.fn = self.lib.gss_sort_u64_descending
+            if kind not in ("u32", "u64"):
+                raise NotImplementedError("descending order is exported for u32 / u64 keys")
+            self.fn = getattr(self.lib, f"gss_sort_{'pairs_' if pairs else ''}{kind}_descending")
         else:
             self.fn = getattr(self.lib, f"gss_sort_{'pairs_' if pairs else ''}{kind}")
 

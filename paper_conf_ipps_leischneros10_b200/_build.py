@@ -89,5 +89,27 @@ def build(force: bool = False, verbose: bool = False) -> str:
     return LIB
 
 
+CXX_TEST_SRC = os.path.join(ROOT, "tests", "cxx", "custom_less.cu")
+CXX_TEST_LIB = os.path.join(ROOT, "tests", "cxx", "libgss_cxx_test.so")
+
+
+def build_cxx_test(force: bool = False, verbose: bool = False) -> str:
+    """Compile tests/cxx/custom_less.cu (include/gss.hpp with user comparators, the comparator-only
+    contract of P:52-54) into tests/cxx/libgss_cxx_test.so for sm_100a."""
+    dep = [CXX_TEST_SRC, os.path.join(ROOT, "include", "gss.hpp")] + deps()
+    if not force and os.path.exists(CXX_TEST_LIB) and all(os.path.getmtime(d) <= os.path.getmtime(CXX_TEST_LIB)
+                                                          for d in dep):
+        return CXX_TEST_LIB
+    cmd = [NVCC, *FLAGS, "-I", nccl_dirs()[0], "-shared", "-o", CXX_TEST_LIB + ".tmp", CXX_TEST_SRC]
+    r = subprocess.run(cmd, capture_output=True, text=True)
+    if r.returncode != 0:
+        sys.stderr.write(r.stderr[-4000:])
+        raise RuntimeError(f"nvcc failed for {CXX_TEST_SRC}")
+    os.replace(CXX_TEST_LIB + ".tmp", CXX_TEST_LIB)
+    if verbose:
+        print(f"built {CXX_TEST_LIB}")
+    return CXX_TEST_LIB
+
+
 if __name__ == "__main__":
     build(force="--force" in sys.argv, verbose=True)

@@ -59,6 +59,18 @@ gss_status gss_sort_u64_descending(const uint64_t* ki, uint64_t* ko, size_t n, v
                                    const gss_params* p) {
   return drive<uint64_t, NoVal, Greater>(io_dev(ki, nullptr, ko, nullptr), n, t, tb, s, p, MODE_SORT, false);
 }
+gss_status gss_sort_u32_descending(const uint32_t* ki, uint32_t* ko, size_t n, void* t, size_t* tb, void* s,
+                                   const gss_params* p) {
+  return drive<uint32_t, NoVal, Greater>(io_dev(ki, nullptr, ko, nullptr), n, t, tb, s, p, MODE_SORT, false);
+}
+gss_status gss_sort_pairs_u32_descending(const uint32_t* ki, const uint32_t* vi, uint32_t* ko, uint32_t* vo, size_t n,
+                                         void* t, size_t* tb, void* s, const gss_params* p) {
+  return drive<uint32_t, uint32_t, Greater>(io_dev(ki, vi, ko, vo), n, t, tb, s, p, MODE_SORT, false);
+}
+gss_status gss_sort_pairs_u64_descending(const uint64_t* ki, const uint64_t* vi, uint64_t* ko, uint64_t* vo, size_t n,
+                                         void* t, size_t* tb, void* s, const gss_params* p) {
+  return drive<uint64_t, uint64_t, Greater>(io_dev(ki, vi, ko, vo), n, t, tb, s, p, MODE_SORT, false);
+}
 
 gss_status gss_sort_f32(const float* ki, float* ko, size_t n, void* t, size_t* tb, void* s, const gss_params* p) {
   return drive<float, NoVal, TotalLess>(io_dev(ki, nullptr, ko, nullptr), n, t, tb, s, p, MODE_SORT, false);

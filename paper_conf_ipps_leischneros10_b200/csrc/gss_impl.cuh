@@ -663,6 +663,9 @@ inline IO io_host(const void* kin, const void* vin, void* kout, void* vout) {
   X(uint32_t, uint32_t, Less)    \
   X(uint64_t, uint64_t, Less)    \
   X(uint64_t, NoVal, Greater)    \
+  X(uint32_t, NoVal, Greater)    \
+  X(uint32_t, uint32_t, Greater) \
+  X(uint64_t, uint64_t, Greater) \
   X(float, NoVal, TotalLess)     \
   X(double, NoVal, TotalLess)
 #ifndef GSS_INSTANTIATING

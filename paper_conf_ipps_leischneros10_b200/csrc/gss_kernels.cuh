@@ -945,7 +945,6 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   constexpr int NW = kScatterThreads / 32;
   using SM = ScatterBulkSmem<Key, Val, IdT>;
   constexpr uint32_t A = SM::A;
-  static_assert(sizeof(Val) == sizeof(Key) || !kHasVal<Val>, "values have the key's width");
   uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);       // next global index of each id (this tile)
   uint32_t* rstart = gbase + kmax;                                // staging slot of each id's run (this chunk)
   uint32_t* rlen = rstart + kmax;                                 // run length of each id (this chunk)
@@ -1096,27 +1095,22 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     const uint32_t sk_s = (uint32_t)__cvta_generic_to_shared(sk);
     uint32_t sv_s = 0;
     if constexpr (kHasVal<Val>) sv_s = (uint32_t)__cvta_generic_to_shared(sv);
-    // one piece: dst[0..cnt) <- staging[so..so+cnt): head / tail elements by
-    // this thread, the 16-byte-aligned middle by one bulk copy
-    auto put = [&](Key* dk, Val* dv, uint32_t so, uint32_t cnt) {
-      const uint32_t mis = (uint32_t)(reinterpret_cast<uintptr_t>(dk) & 15u) / (uint32_t)sizeof(Key);
-      uint32_t head = min(cnt, (A - mis) & (A - 1));
+    // one piece of one array: dst[0..cnt) <- staging[so..so+cnt): head / tail
+    // elements by this thread, the 16-byte-aligned middle by one bulk copy
+    auto put1 = [&](auto* d, const auto* stg, uint32_t stg_s, uint32_t so, uint32_t cnt) {
+      constexpr uint32_t W = (uint32_t)sizeof(*d), AW = 16u / W;
+      const uint32_t mis = (uint32_t)(reinterpret_cast<uintptr_t>(d) & 15u) / W;
+      uint32_t head = min(cnt, (AW - mis) & (AW - 1));
       // the staging slot matches the destination modulo 16 bytes (else: element by element)
-      if (((sk_s + (so + head) * (uint32_t)sizeof(Key)) & 15u) != 0) head = cnt;
-      const uint32_t mid_end = head + ((cnt - head) & ~(A - 1));
-      for (uint32_t h = 0; h < head; h++) {
-        dk[h] = sk[so + h];
-        if constexpr (kHasVal<Val>) dv[h] = sv[so + h];
-      }
-      if (mid_end > head) {
-        bulk_s2g(dk + head, sk_s + (so + head) * (uint32_t)sizeof(Key), (mid_end - head) * (uint32_t)sizeof(Key));
-        if constexpr (kHasVal<Val>)
-          bulk_s2g(dv + head, sv_s + (so + head) * (uint32_t)sizeof(Val), (mid_end - head) * (uint32_t)sizeof(Val));
-      }
-      for (uint32_t h = mid_end; h < cnt; h++) {
-        dk[h] = sk[so + h];
-        if constexpr (kHasVal<Val>) dv[h] = sv[so + h];
-      }
+      if (((stg_s + (so + head) * W) & 15u) != 0) head = cnt;
+      const uint32_t mid_end = head + ((cnt - head) & ~(AW - 1));
+      for (uint32_t h = 0; h < head; h++) d[h] = stg[so + h];
+      if (mid_end > head) bulk_s2g(d + head, stg_s + (so + head) * W, (mid_end - head) * W);
+      for (uint32_t h = mid_end; h < cnt; h++) d[h] = stg[so + h];
+    };
+    auto put = [&](Key* dk, Val* dv, uint32_t so, uint32_t cnt) {
+      put1(dk, sk, sk_s, so, cnt);
+      if constexpr (kHasVal<Val>) put1(dv, sv, sv_s, so, cnt);
     };
     for (uint32_t j = 0; j < per; j++) {
       const uint32_t id = i0 + j;

@@ -92,3 +92,13 @@ def test_product_does_not_import_oracle():
             if f.endswith((".py", ".cu", ".cuh", ".h")):
                 txt = open(os.path.join(dirpath, f)).read()
                 assert "import oracle" not in txt and "from oracle" not in txt and "oracle.h" not in txt, f
+
+
+
+def test_cxx_template_header_builds_and_exports():
+    """include/gss.hpp instantiated with user comparators (tests/cxx/custom_less.cu) compiles
+    for sm_100a and loads without a GPU."""
+    from paper_conf_ipps_leischneros10_b200 import _build
+    lib = ctypes.CDLL(_build.build_cxx_test())
+    for name in ("cxx_sort_residue_u64", "cxx_sort_pairs_desc_u32_u64"):
+        assert hasattr(lib, name)

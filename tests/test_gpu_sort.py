@@ -552,3 +552,68 @@ def test_float_total_order(gss, oracle_mod, width):
     assert np.all(nan[:int((nan & sgn).sum())]) and np.all(nan[n - int((nan & ~sgn).sum()):])
     z = np.flatnonzero(y == 0)
     assert np.all(np.diff(sgn[z].astype(np.int8)) <= 0)
+
+
+
+# ---------------------------------------------------------------------------
+# Comparator-only contract: descending order for every kind, and
+# include/gss.hpp instantiated with user comparators (tests/cxx/custom_less.cu)
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist", ["uniform", "dd", "and4"])
+def test_descending_all_kinds(gss, oracle_mod, width, pairs, dist):
+    n = (1 << 20) + 99
+    x = inputs.keys(dist, n, width, seed=21)
+    v = inputs.values(n, width) if pairs else None
+    ok, _, _ = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=4096))
+    ko, vo = gss.sort(to_dev(x), to_dev(v) if pairs else None, descending=True, M=4096)
+    np.testing.assert_array_equal(to_host(ko), ok[::-1])
+    if pairs:
+        check_pairs(x, to_host(vo), ok[::-1])
+
+
+@pytest.fixture(scope="module")
+def cxx_lib():
+    import ctypes
+    from paper_conf_ipps_leischneros10_b200 import _build
+    lib = ctypes.CDLL(_build.build_cxx_test())
+    vp, sz = ctypes.c_void_p, ctypes.c_size_t
+    lib.cxx_sort_residue_u64.restype = ctypes.c_int
+    lib.cxx_sort_residue_u64.argtypes = [vp, vp, sz, vp, ctypes.POINTER(sz), vp]
+    lib.cxx_sort_pairs_desc_u32_u64.restype = ctypes.c_int
+    lib.cxx_sort_pairs_desc_u32_u64.argtypes = [vp, vp, vp, vp, sz, vp, ctypes.POINTER(sz), vp]
+    return lib
+
+
+def _cxx_call(fn, head):
+    import ctypes
+    tb = ctypes.c_size_t(0)
+    assert fn(*head, None, ctypes.byref(tb), None) == 0
+    temp = torch.empty(max(tb.value, 1), dtype=torch.uint8, device="cuda")
+    s = torch.cuda.current_stream().cuda_stream
+    assert fn(*head, ctypes.c_void_p(temp.data_ptr()), ctypes.byref(tb), s) == 0
+    torch.cuda.synchronize()
+
+
+@pytest.mark.parametrize("n", [1000, (1 << 20) + 7])
+def test_gss_hpp_user_comparators(gss, cxx_lib, n):
+    import ctypes
+    p = lambda t: ctypes.c_void_p(t.data_ptr())  # noqa: E731
+    # u64 keys by residue mod 1000003: equivalent keys form runs in any order
+    x = inputs.keys("uniform", n, 64, seed=5)
+    kin, kout = to_dev(x), torch.empty(n, dtype=torch.uint64, device="cuda")
+    _cxx_call(cxx_lib.cxx_sort_residue_u64, (p(kin), p(kout), n))
+    y = to_host(kout)
+    r = y % np.uint64(1000003)
+    assert np.all(r[1:] >= r[:-1])
+    np.testing.assert_array_equal(np.sort(y), np.sort(x))
+    # u32 keys, u64 values, descending: a key/value width pair libgss.so does not export
+    k32 = inputs.keys("and2", n, 32, seed=6)
+    v64 = np.arange(n, dtype=np.uint64)
+    ki, vi = to_dev(k32), to_dev(v64)
+    ko, vo = torch.empty_like(ki), torch.empty_like(vi)
+    _cxx_call(cxx_lib.cxx_sort_pairs_desc_u32_u64, (p(ki), p(vi), p(ko), p(vo), n))
+    got_k, got_v = to_host(ko), to_host(vo).astype(np.int64)
+    np.testing.assert_array_equal(got_k, np.sort(k32)[::-1])
+    np.testing.assert_array_equal(np.sort(got_v), np.arange(n))
+    np.testing.assert_array_equal(k32[got_v], got_k)
