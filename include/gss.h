@@ -56,7 +56,7 @@ typedef enum gss_status {
   GSS_ERROR_TEMP_TOO_SMALL = 2,  /* *temp_bytes smaller than the query returned         */
   GSS_ERROR_NOT_SUPPORTED = 3,   /* n >= 2^32, or device is not sm_100                   */
   GSS_ERROR_CUDA = 4,            /* a launch or runtime call failed                      */
-  GSS_ERROR_NCCL = 5,            /* reserved for the distributed layer                   */
+  GSS_ERROR_NCCL = 5,            /* a collective of gss_dist_* failed                    */
   GSS_ERROR_CAPACITY = 6         /* an output capacity is smaller than the result        */
 } gss_status;
 
@@ -101,7 +101,9 @@ typedef struct gss_params {
   uint32_t fill_div;        /* adaptive rule divisor f (R29); 0 -> 4              */
   uint64_t seed;            /* sampling seed (R2); 0 -> 5489                               */
   uint32_t flags;           /* GSS_FLAG_* below                                            */
-  uint32_t reserved;
+  uint32_t cls_arrays;      /* Phase-2 counter arrays per CTA of 8 warps: 1, 2, 4 or 8; 0 ->
+                               8, one per warp (the paper splits counter contention over 8
+                               arrays; ablation SURVEY NEXT-4 iii)               */
   gss_stats* stats;         /* optional host pointer: the call syncs and fills it          */
   gss_profiler* profiler;   /* optional: CUDA-event time of every launch                   */
 } gss_params;
@@ -132,6 +134,10 @@ typedef struct gss_params {
                                       call needing larger windows) allocates and registers the
                                       windows collectively (ncclMemAlloc +
                                       ncclCommWindowRegister)                                 */
+#define GSS_FLAG_BITONIC_NET 128u  /* u64 keys: each thread of the in-SM sort sorts its 16 keys
+                                      with a bitonic network instead of Batcher's odd-even
+                                      merge network (the paper's comparison, P:339-341;
+                                      ablation SURVEY NEXT-4 iv); ignored for other kinds    */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets of two or more warps with one more
                                       sample-sort split inside the SM + warp merge sorts of
                                       packed segments; ablation: on B200 its

@@ -39,7 +39,7 @@ class _Stats(ctypes.Structure):
 class _Params(ctypes.Structure):
     _fields_ = [("k", _u32), ("oversample", _u32), ("small_threshold", _u64), ("tile", _u32),
                 ("max_levels", _u32), ("k_policy", _u32), ("fill_div", _u32), ("seed", _u64), ("flags", _u32),
-                ("reserved", _u32), ("stats", ctypes.POINTER(_Stats)), ("profiler", _vp)]
+                ("cls_arrays", _u32), ("stats", ctypes.POINTER(_Stats)), ("profiler", _vp)]
 
 
 @dataclass
@@ -165,7 +165,7 @@ class Profiler:
 
 
 def _params(k=None, M=None, a=None, tile=None, seed=None, k_policy=None, fill_div=None, max_levels=None,
-            flags=0, stats=None, profiler=None):
+            flags=0, stats=None, profiler=None, cls_arrays=None):
     p = _Params()
     p.k = k or 0
     p.small_threshold = M or 0
@@ -176,6 +176,7 @@ def _params(k=None, M=None, a=None, tile=None, seed=None, k_policy=None, fill_di
     p.fill_div = fill_div or 0
     p.max_levels = max_levels or 0
     p.flags = flags
+    p.cls_arrays = cls_arrays or 0
     if stats is not None:
         p.stats = ctypes.pointer(stats)
     if profiler is not None:

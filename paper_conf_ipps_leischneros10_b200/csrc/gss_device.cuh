@@ -124,6 +124,7 @@ struct Ctx {
   const Key* given_spl;              // MODE_PARTITION_BY
   uint32_t given_nspl;
   uint32_t given_eq;                 // MODE_PARTITION_BY in equality mode (ids 2b / 2b+1)
+  uint32_t cls_arrays;               // Phase-2 counter arrays per CTA (8 = one per warp)
   const RemoteSeg* remote;           // MODE_PARTITION_BY, phase 2: destinations on other GPUs
   uint32_t nremote;
   uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
@@ -317,7 +318,7 @@ __device__ __forceinline__ void oem_sort(Key* k, Val* v, Cmp less) {
 
 // Bitonic sort network on k[0 .. N) (N a power of two), compile-time indices:
 // the alternative the paper measured against odd-even merge;
-// selected with -DGSS_THREAD_NET=1 (ablation).
+// selected with GSS_FLAG_BITONIC_NET (ablation).
 template <int N, class Key, class Val, class Cmp>
 __device__ __forceinline__ void bitonic_sort_regs(Key* k, Val* v, Cmp less) {
 #pragma unroll
@@ -336,12 +337,10 @@ __device__ __forceinline__ void bitonic_sort_regs(Key* k, Val* v, Cmp less) {
   }
 }
 
-#ifndef GSS_THREAD_NET
-#define GSS_THREAD_NET 0   // 0: Batcher odd-even merge sort (default), 1: bitonic sort
-#endif
-template <int N, class Key, class Val, class Cmp>
+// BITONIC: the ablation GSS_FLAG_BITONIC_NET (runtime flag, u64 keys only)
+template <int N, bool BITONIC, class Key, class Val, class Cmp>
 __device__ __forceinline__ void thread_sort_net(Key* k, Val* v, Cmp less) {
-  if constexpr (GSS_THREAD_NET == 1) bitonic_sort_regs<N>(k, v, less);
+  if constexpr (BITONIC) bitonic_sort_regs<N>(k, v, less);
   else oem_sort<0, N>(k, v, less);
 }
 
@@ -382,7 +381,7 @@ constexpr int sort_items() {
 // current a -- the same key value.  With values the stand-ins must never be
 // taken: A wins ties (B's stand-in is >= a, so A is taken) and A carries one
 // index test.  Either way the merge loop has no per-step bounds tests.
-template <class Key, class Val, int NT, class Cmp, int ITEMS_ = sort_items<Key, Val>()>
+template <class Key, class Val, int NT, class Cmp, int ITEMS_ = sort_items<Key, Val>(), bool BITONIC = false>
 struct CtaSort {
   static constexpr int ITEMS = ITEMS_;
   static constexpr int C = NT * ITEMS;
@@ -685,9 +684,9 @@ struct CtaSort {
       }
       if constexpr (KV) {
         if (stable_path) transposition_sort<ITEMS>(k, v, less);
-        else thread_sort_net<ITEMS>(k, v, less);
+        else thread_sort_net<ITEMS, BITONIC>(k, v, less);
       } else {
-        thread_sort_net<ITEMS>(k, v, less);
+        thread_sort_net<ITEMS, BITONIC>(k, v, less);
       }
     }
     __syncwarp();

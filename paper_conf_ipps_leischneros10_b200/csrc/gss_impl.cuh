@@ -69,7 +69,7 @@ inline gss_status device_info(DeviceInfo* out) {
 
 // Resolved parameters.
 struct Cfg {
-  uint32_t k, a, T, L, k_policy, fill_div, flags, kmax, nclass;
+  uint32_t k, a, T, L, k_policy, fill_div, flags, kmax, nclass, cls_arrays;
   uint64_t M, seed;
   uint32_t class_cap[kNumClasses];
 };
@@ -111,6 +111,8 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   c->fill_div = p.fill_div ? p.fill_div : 4;
   c->seed = p.seed ? p.seed : 5489;
   c->flags = p.flags;
+  c->cls_arrays = p.cls_arrays ? p.cls_arrays : 8;
+  if (c->cls_arrays != 1 && c->cls_arrays != 2 && c->cls_arrays != 4 && c->cls_arrays != 8) return GSS_ERROR_INVALID_VALUE;
   // size classes (R8): class i = buckets a CTA of class_warps(i) warps sorts
   c->nclass = kNumClasses;
   for (int i = 0; i < kNumClasses; i++) c->class_cap[i] = (uint32_t)(class_warps(i) * 32 * small_items<Key, Val>());
@@ -292,6 +294,7 @@ struct Engine {
     c.cap_spl = lay.cap_spl; c.cap_copy = lay.cap_copy; c.cap_ovf = lay.cap_ovf;
     c.cap_fb = lay.cap_fb;
     c.seed = cfg.seed;
+    c.cls_arrays = cfg.cls_arrays;
     return c;
   }
 
@@ -314,11 +317,15 @@ struct Engine {
       return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, ns, smem, s>>>(c, (uint32_t)cls); });
     }
     auto kern = k_small_block<Key, Val, IdT, Cmp>;
+    if constexpr (sizeof(Key) == 8 && !kHasVal<Val> && std::is_same<Cmp, Less>::value) {
+      if (cfg.flags & GSS_FLAG_BITONIC_NET) kern = k_small_block<Key, Val, IdT, Cmp, true>;   // ablation
+    }
     const size_t smem = block_sort_smem_bytes<Key, Val>(nt);
     GSS_TRY(set_smem(kern, block_sort_smem_bytes<Key, Val>(kSmallMaxThreads)));
-    static GridCache grid[kNumClasses + 1];
-    int g = grid[cls].get(di.dev);
-    if (!g) { g = grid_for(kern, nt, smem, di.sms); grid[cls].put(di.dev, g); }
+    static GridCache grid[2][kNumClasses + 1];
+    const int gv = (cfg.flags & GSS_FLAG_BITONIC_NET) ? 1 : 0;
+    int g = grid[gv][cls].get(di.dev);
+    if (!g) { g = grid_for(kern, nt, smem, di.sms); grid[gv][cls].put(di.dev, g); }
     return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, nt, smem, s>>>(c, (uint32_t)cls); });
   }
 
@@ -586,7 +593,7 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
       key.n = n;
       key.p[0] = io.kin; key.p[1] = io.kout; key.p[2] = io.vin; key.p[3] = io.vout; key.p[4] = temp;
       key.cfg[0] = cfg.k; key.cfg[1] = cfg.a; key.cfg[2] = cfg.T; key.cfg[3] = cfg.L; key.cfg[4] = cfg.k_policy;
-      key.cfg[5] = cfg.fill_div; key.cfg[6] = cfg.flags; key.cfg[7] = (uint32_t)cfg.M;
+      key.cfg[5] = cfg.fill_div | (cfg.cls_arrays << 24); key.cfg[6] = cfg.flags; key.cfg[7] = (uint32_t)cfg.M;
       key.seed = cfg.seed;
       cudaGraphExec_t exec = graph_lookup(key);
       if (!exec) {

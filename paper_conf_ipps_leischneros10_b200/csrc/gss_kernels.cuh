@@ -397,12 +397,10 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
   const uint32_t per = (nt + gridDim.x - 1) / gridDim.x;
   const uint32_t t0 = blockIdx.x * per, t1 = min(nt, t0 + per);
   // Counter arrays (the paper splits contention over 8 arrays).  Default: one per warp (8 per CTA,
-  // 32 threads each, as in the paper); -DGSS_CLS_NARR=1/2/4 shares arrays between warps (SURVEY NEXT-4 iii).
-#ifndef GSS_CLS_NARR
-#define GSS_CLS_NARR NW
-#endif
-  static_assert(NW % GSS_CLS_NARR == 0, "counter arrays must divide the warps");
-  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + (w / (NW / GSS_CLS_NARR)) * kmax);
+  // 32 threads each, as in the paper); gss_params.cls_arrays = 1/2/4 shares arrays between warps (SURVEY
+  // NEXT-4 iii, an ablation)
+  const uint32_t narr = c.cls_arrays;                          // 1, 2, 4 or 8 (= NW)
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wcnt + (w / (NW / narr)) * kmax);
   const uint32_t tree_s = (uint32_t)__cvta_generic_to_shared(tree);
   // node j of levels 5..7 is read by this lane at rep_b + 128 j
   const uint32_t rep_b = (uint32_t)__cvta_generic_to_shared(rep) - (1u << kTopLevels) * 128u +
@@ -422,7 +420,7 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
       }
       cur = b;
     }
-    for (uint32_t j = threadIdx.x; j < NW * kmax; j += kClsThreads) wcnt[j] = 0;
+    for (uint32_t j = threadIdx.x; j < narr * kmax; j += kClsThreads) wcnt[j] = 0;
     __syncthreads();
     const uint32_t tl = t - B.tile_start;
     const uint32_t beg = B.lo + tl * c.T;
@@ -445,7 +443,7 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
     for (uint32_t id = threadIdx.x; id < B.K; id += kClsThreads) {
       uint32_t s = 0;
 #pragma unroll
-      for (int q = 0; q < NW; q++) s += wcnt[q * kmax + id];
+      for (int q = 0; q < NW; q++) s += (uint32_t)q < narr ? wcnt[q * kmax + id] : 0u;
       hist[id * B.ntiles + tl] = s;
     }
   }
@@ -1625,12 +1623,12 @@ __host__ __device__ constexpr size_t block_sort_smem_bytes(int nt) {
 #ifndef GSS_SMALL_CPASYNC
 #define GSS_SMALL_CPASYNC 1   // 8-byte keys: 4.83 vs 4.96 ms (2^28 u64), pairs 4.45 vs 4.57; 4-byte copies lose (2.15 vs 1.58)
 #endif
-template <class Key, class Val, class IdT, class Cmp>
+template <class Key, class Val, class IdT, class Cmp, bool BITONIC = false>
 __global__ void __launch_bounds__(kSmallMaxThreads, 1)
     k_small_block(Ctx<Key, Val, IdT> c, uint32_t cls) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   constexpr int ITEMS = small_items<Key, Val>();
-  using Sorter = CtaSort<Key, Val, kSmallMaxThreads, Cmp, ITEMS>;
+  using Sorter = CtaSort<Key, Val, kSmallMaxThreads, Cmp, ITEMS, BITONIC>;
   const int nt = (int)blockDim.x;
   Key* sk = reinterpret_cast<Key*>(smem_raw);
   Val* sv = reinterpret_cast<Val*>(smem_raw + (size_t)padded_len(nt * ITEMS) * sizeof(Key));

@@ -617,3 +617,31 @@ def test_gss_hpp_user_comparators(gss, cxx_lib, n):
     np.testing.assert_array_equal(got_k, np.sort(k32)[::-1])
     np.testing.assert_array_equal(np.sort(got_v), np.arange(n))
     np.testing.assert_array_equal(k32[got_v], got_k)
+
+
+# ---------------------------------------------------------------------------
+# The paper's design alternatives as runtime ablations, each
+# against the oracle: (iii) fewer Phase-2 counter arrays per CTA,
+# (iv) bitonic instead of odd-even merge networks in the in-SM sort
+# (P:339-341); (i) recompute ids and (ii) the direct scatter are above.
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("variant", [dict(cls_arrays=1), dict(cls_arrays=2), dict(cls_arrays=4),
+                                     dict(flags=128), dict(flags=32), dict(flags=128 | 16)])
+def test_ablation_variants_vs_oracle(gss, oracle_mod, width, pairs, variant):
+    n = (1 << 21) + 333
+    x = inputs.keys("and3", n, width, seed=31)
+    v = inputs.values(n, width) if pairs else None
+    M = 4096
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=M), log=True)
+    graph = bool(variant.get("flags", 0) & 16)                 # the graph path ignores statistics
+    if graph:
+        ko, vo = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=M, **variant)
+        st = None
+    else:
+        ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=M, stats=True, **variant)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if pairs:
+        check_pairs(x, to_host(vo), ok)
+    if st is not None:
+        assert_levels_match(st, recs)
