@@ -236,7 +236,8 @@ __device__ __forceinline__ uint64_t block_sum_u64(uint64_t x, unsigned long long
 // through shared memory.  Shared layout: element i at i + i/16 (conflict-free
 // blocked access).
 // --------------------------------------------------------------------------
-__host__ __device__ constexpr int padded_len(int c) { return c + c / 16 + 1; }
+// rounded up to 4 slots so that a value array placed after the key array stays 16-byte aligned
+__host__ __device__ constexpr int padded_len(int c) { return (c + c / 16 + 1 + 3) & ~3; }
 __device__ __forceinline__ int phys(int i) { return i + (i >> 4); }
 
 #ifndef GSS_FAST_KV
