@@ -82,6 +82,7 @@ typedef struct gss_stats {
   uint64_t eq_elems;
   uint64_t overflow_buckets;    /* buckets finished by the fallback after max_levels     */
   uint64_t overflow_elems;
+  uint64_t cluster_buckets;     /* buckets sorted by a thread-block cluster (GSS_FLAG_CLUSTER_SORT) */
 } gss_stats;
 
 typedef struct gss_profiler gss_profiler;
@@ -138,6 +139,11 @@ typedef struct gss_params {
                                       with a bitonic network instead of Batcher's odd-even
                                       merge network (the paper's comparison, P:339-341;
                                       ablation SURVEY NEXT-4 iv); ignored for other kinds    */
+#define GSS_FLAG_CLUSTER_SORT 256u /* buckets above one CTA's shared-memory capacity (up to M)
+                                      are sorted by a cluster of 8 CTAs through distributed
+                                      shared memory (the on-chip answer to the
+                                      paper's quicksort tier below M = 2^17); the
+                                      default M becomes the cluster capacity (8x the CTA's)  */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets of two or more warps with one more
                                       sample-sort split inside the SM + warp merge sorts of
                                       packed segments; ablation: on B200 its

@@ -33,7 +33,7 @@ class _Stats(ctypes.Structure):
     _fields_ = [("levels", _u32), ("launches", _u32), ("levels_launched", _u32), ("error_flags", _u32),
                 ("split_elems", _u64 * 16), ("split_buckets", _u64 * 16), ("small_buckets", _u64),
                 ("small_elems", _u64), ("max_small", _u64), ("eq_buckets", _u64), ("eq_elems", _u64),
-                ("overflow_buckets", _u64), ("overflow_elems", _u64)]
+                ("overflow_buckets", _u64), ("overflow_elems", _u64), ("cluster_buckets", _u64)]
 
 
 class _Params(ctypes.Structure):
@@ -57,13 +57,14 @@ class Stats:
     eq_elems: int
     overflow_buckets: int
     overflow_elems: int
+    cluster_buckets: int = 0
 
     @staticmethod
     def _from(s: _Stats) -> "Stats":
         L = 16
         return Stats(s.levels, s.launches, s.levels_launched, s.error_flags, list(s.split_elems[:L]),
                      list(s.split_buckets[:L]), s.small_buckets, s.small_elems, s.max_small, s.eq_buckets,
-                     s.eq_elems, s.overflow_buckets, s.overflow_elems)
+                     s.eq_elems, s.overflow_buckets, s.overflow_elems, s.cluster_buckets)
 
 
 _LIB = None

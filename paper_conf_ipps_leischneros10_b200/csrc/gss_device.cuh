@@ -46,6 +46,13 @@ struct Less {
 struct Greater {
   template <class T> __device__ __forceinline__ bool operator()(const T& a, const T& b) const { return b < a; }
 };
+// Orders under which equivalent keys are bit-identical, so that a copy of a
+// key is indistinguishable from the key (the in-SM sort's bounds-free merge
+// and padding rely on it; any other comparator takes the safe paths).
+template <class Cmp> struct BitwiseOrder : std::false_type {};
+template <> struct BitwiseOrder<Less> : std::true_type {};
+template <> struct BitwiseOrder<Greater> : std::true_type {};
+
 // IEEE-754 total order for floating-point keys: -NaN < -inf < ... < -0 < +0 <
 // ... < +inf < +NaN, i.e. a strict weak (in fact total) order on bit patterns.
 struct TotalLess {
@@ -61,6 +68,7 @@ struct TotalLess {
     return rank(a) < rank(b);
   }
 };
+template <> struct BitwiseOrder<TotalLess> : std::true_type {};     // rank() is a bijection on bit patterns
 
 // A bucket being split at some level (one row of the paper's k x p table
 // per tile).
@@ -103,6 +111,7 @@ struct Counters {
   uint32_t small_count[kNumClasses];
   uint32_t copy_count, ovf_count, err, fb_count;   // fb: buckets the in-SM split hands to the block sort
   unsigned long long small_elems, max_small, eq_buckets, eq_elems, ovf_elems;
+  uint32_t clus_count, pad_c;                       // buckets for the cluster-wide sort (GSS_FLAG_CLUSTER_SORT)
 };
 
 // Everything a kernel needs, passed by value.
@@ -120,6 +129,7 @@ struct Ctx {
   Item* copy;
   Item* ovf;
   Item* fb;
+  Item* clus;                        // buckets above one CTA's capacity, sorted by a thread-block cluster
   uint32_t* scan_part;
   const Key* given_spl;              // MODE_PARTITION_BY
   uint32_t given_nspl;
@@ -129,7 +139,7 @@ struct Ctx {
   uint32_t nremote;
   uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
   uint32_t recompute;                // GSS_FLAG_RECOMPUTE_IDS: no stored ids, Phase 4 re-descends
-  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb;
+  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb, cap_clus;
   uint32_t cap_small[kNumClasses];
   uint32_t class_cap[kNumClasses];
   uint64_t seed;
@@ -388,6 +398,10 @@ struct CtaSort {
   static constexpr int C = NT * ITEMS;
   static constexpr int PL = padded_len(C);
   static constexpr bool KV = kHasVal<Val>;
+  // SAFE: the merge never takes a stand-in key and partial threads keep their
+  // items apart from the pads -- needed with values, and with comparators whose
+  // equivalent keys need not be bit-identical (user comparators, gss.hpp)
+  static constexpr bool SAFE = KV || !BitwiseOrder<Cmp>::value;
   // keys-only unsigned keys under operator<: the merge step in PTX
   static constexpr bool kFastMerge = !KV && std::is_same<Cmp, Less>::value && std::is_unsigned<Key>::value &&
                                      (sizeof(Key) == 4 || sizeof(Key) == 8);
@@ -500,7 +514,7 @@ struct CtaSort {
     // pair width w = max(aLen, ...) is a power of two, the same for every lane
     // of the round): no data-dependent trip count, no divergence.
     const int w = aLen;                                       // aLen == w for every pair with a B run
-    if constexpr (KV) {
+    if constexpr (SAFE) {
       // number of A keys among the first diag outputs, A first on ties:
       // smallest j in [lo, hi) with B[diag-1-j] < A[j], else hi
       const int lo = max(0, diag - bLen), hi = min(diag, aLen);
@@ -571,7 +585,7 @@ struct CtaSort {
 #pragma unroll
     for (int i = 0; i < ITEMS; i++) {
       bool p;
-      if constexpr (KV) p = (xa < ae) && !less(kb, ka);
+      if constexpr (SAFE) p = (xa < ae) && !less(kb, ka);
       else p = less(ka, kb);
       k[i] = p ? ka : kb;
       if constexpr (KV) v[i] = p ? va : vb;
@@ -668,7 +682,7 @@ struct CtaSort {
 #pragma unroll
         for (int i = 1; i < ITEMS; i++)
           if (i < cnt && less(mx, k[i])) { mx = k[i]; vmx = v[i]; }
-        if constexpr (KV) {
+        if constexpr (SAFE) {
           int reps = 0;
 #pragma unroll
           for (int i = 0; i < ITEMS; i++)
@@ -683,7 +697,7 @@ struct CtaSort {
           }
         }
       }
-      if constexpr (KV) {
+      if constexpr (SAFE) {
         if (stable_path) transposition_sort<ITEMS>(k, v, less);
         else thread_sort_net<ITEMS, BITONIC>(k, v, less);
       } else {

@@ -84,7 +84,8 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   gss_params p{};
   if (up) p = *up;
   c->a = p.oversample ? p.oversample : 30;
-  const uint32_t cap = max_small_capacity<Key, Val>();
+  // GSS_FLAG_CLUSTER_SORT: buckets up to a thread-block cluster's capacity are final (NEXT-2)
+  const uint32_t cap = (p.flags & GSS_FLAG_CLUSTER_SORT) ? cluster_capacity<Key, Val>() : max_small_capacity<Key, Val>();
   c->M = p.small_threshold ? p.small_threshold : cap;
   if (c->M > cap) return GSS_ERROR_INVALID_VALUE;
   // default k (R29): 256, raised to 512 / 1024 when two levels of 256 would
@@ -116,7 +117,7 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   // size classes (R8): class i = buckets a CTA of class_warps(i) warps sorts
   c->nclass = kNumClasses;
   for (int i = 0; i < kNumClasses; i++) c->class_cap[i] = (uint32_t)(class_warps(i) * 32 * small_items<Key, Val>());
-  if (c->class_cap[kNumClasses - 1] != cap) return GSS_ERROR_NOT_SUPPORTED;
+  if (c->class_cap[kNumClasses - 1] != max_small_capacity<Key, Val>()) return GSS_ERROR_NOT_SUPPORTED;
   c->kmax = std::max<uint32_t>(std::max(c->k, kmin_given), 4u);
   // levels: expected depth with children up to 2x the mean, plus one spare level
   if (p.max_levels) {
@@ -138,8 +139,8 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
 template <class Key, class Val, class IdT>
 struct Layout {
   size_t off_cnt, off_ktmp, off_vtmp, off_ids, off_bk[2], off_tb[2], off_hist[2], off_spl[2], off_small[kNumClasses],
-      off_copy, off_ovf, off_fb, off_scan, off_hin_k, off_hin_v, off_hout_k, off_hout_v, total;
-  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb, cap_small[kNumClasses];
+      off_copy, off_ovf, off_fb, off_clus, off_scan, off_hin_k, off_hin_v, off_hout_k, off_hout_v, total;
+  uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb, cap_clus, cap_small[kNumClasses];
 
   void compute(uint64_t n, const Cfg& c, int mode, bool host_io) {
     const uint64_t M = mode == MODE_SORT ? c.M : 0;
@@ -156,6 +157,8 @@ struct Layout {
     cap_copy = (uint32_t)(n / c.T + n / (c.class_cap[kNumClasses - 1] + 1) + 2);
     cap_ovf = cap_buckets;
     cap_fb = mode == MODE_SORT ? (uint32_t)(n / (c.class_cap[0] + 1) + 1) : 1;   // buckets of the split classes
+    cap_clus = (mode == MODE_SORT && M > c.class_cap[kNumClasses - 1])
+                   ? (uint32_t)(n / (c.class_cap[kNumClasses - 1] + 1) + 1) : 1;
     size_t o = 0;
     auto take = [&](size_t bytes) { size_t r = o; o = align_up(o + bytes); return r; };
     off_hin_k = off_hout_k = off_hin_v = off_hout_v = 0;
@@ -181,6 +184,7 @@ struct Layout {
     off_copy = take((size_t)cap_copy * sizeof(Item));
     off_ovf = take((size_t)cap_ovf * sizeof(Item));
     off_fb = take((size_t)cap_fb * sizeof(Item));
+    off_clus = take((size_t)cap_clus * sizeof(Item));
     off_scan = take(kScanCtas * 4);
     total = o;
   }
@@ -280,6 +284,7 @@ struct Engine {
     c.copy = reinterpret_cast<Item*>(base + lay.off_copy);
     c.ovf = reinterpret_cast<Item*>(base + lay.off_ovf);
     c.fb = reinterpret_cast<Item*>(base + lay.off_fb);
+    c.clus = reinterpret_cast<Item*>(base + lay.off_clus);
     c.scan_part = reinterpret_cast<uint32_t*>(base + lay.off_scan);
     c.n = (uint32_t)n;
     c.M = (uint32_t)cfg.M;
@@ -293,6 +298,7 @@ struct Engine {
     c.cap_buckets = lay.cap_buckets; c.cap_tiles = lay.cap_tiles; c.cap_hist = lay.cap_hist;
     c.cap_spl = lay.cap_spl; c.cap_copy = lay.cap_copy; c.cap_ovf = lay.cap_ovf;
     c.cap_fb = lay.cap_fb;
+    c.cap_clus = lay.cap_clus;
     c.seed = cfg.seed;
     c.cls_arrays = cfg.cls_arrays;
     return c;
@@ -403,6 +409,14 @@ struct Engine {
         GSS_TRY(launch(prof, GSS_K_PLAN, s, count, [&] { k_plan<Key, Val, IdT><<<g_plan, kPlanThreads, 0, s>>>(c, l); }));
     }
     if (mode != MODE_SORT) return GSS_SUCCESS;
+    if (cfg.M > cfg.class_cap[kNumClasses - 1]) {
+      // the largest buckets first: thread-block clusters of kClusterCtas CTAs (GSS_FLAG_CLUSTER_SORT)
+      auto kcl = k_small_cluster<Key, Val, IdT, Cmp>;
+      constexpr size_t sm_cl = cluster_smem_bytes<Key, Val>();
+      GSS_TRY(set_smem(kcl, sm_cl));
+      const int g_cl = std::max(1, di.sms / kClusterCtas) * kClusterCtas;
+      GSS_TRY(launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kcl<<<g_cl, kClusterThreads, sm_cl, s>>>(c); }));
+    }
     // in-SM sorts, largest class first (buckets "ordered by size"; R8)
     for (int cls = (int)cfg.nclass - 1; cls >= 0; cls--) GSS_TRY(launch_small(c, cfg, cls, di, s, prof, count));
     if (cfg.flags & GSS_FLAG_SPLIT_SORT) GSS_TRY(launch_small(c, cfg, kNumClasses, di, s, prof, count));
@@ -433,6 +447,7 @@ inline void fill_stats(const Counters& h, uint32_t L, uint32_t launches, gss_sta
   st->eq_elems = h.eq_elems;
   st->overflow_buckets = h.ovf_count;
   st->overflow_elems = h.ovf_elems;
+  st->cluster_buckets = h.clus_count;
 }
 
 // Cache of instantiated launch graphs (GSS_FLAG_GRAPH), keyed by everything

@@ -10,6 +10,8 @@
 // per-level synchronisation.
 #pragma once
 
+#include <cooperative_groups.h>
+
 #include "gss_device.cuh"
 
 namespace gss {
@@ -66,6 +68,13 @@ __global__ void k_init(Ctx<Key, Val, IdT> c) {
   __syncthreads();
   if (threadIdx.x != 0 || c.n == 0) return;
   if (c.mode == MODE_SORT && c.n <= c.M) {
+    c.cnt->small_elems = c.n;
+    c.cnt->max_small = c.n;
+    if (c.n > c.class_cap[kNumClasses - 1]) {                  // GSS_FLAG_CLUSTER_SORT: one cluster sorts it
+      c.clus[0] = Item{0, c.n, c.src0, 0};
+      c.cnt->clus_count = 1;
+      return;
+    }
     uint32_t cls = 0;
     while (cls + 1 < kNumClasses && c.n > c.class_cap[cls]) cls++;
     c.small[cls][0] = Item{0, c.n, c.src0, 0};
@@ -1520,11 +1529,21 @@ __global__ void __launch_bounds__(kPlanThreads) k_plan(Ctx<Key, Val, IdT> c, uin
           atomicAdd(&c.cnt->eq_elems, (unsigned long long)e_el);
         }
       }
+      // buckets above one CTA's capacity (only with GSS_FLAG_CLUSTER_SORT, where M may exceed it): the
+      // cluster-wide sort
+      const bool to_clus = to_small && m > cap_last;
+      if (__any_sync(kFull, to_clus)) {
+        const uint32_t i = warp_append(&c.cnt->clus_count, to_clus ? 1u : 0u);
+        if (to_clus) {
+          if (i < c.cap_clus) c.clus[i] = Item{start, m, db, 0};
+          else atomicOr(&c.cnt->err, 16u);
+        }
+      }
       // in-SM sort lists, one per size class
       uint32_t cls = 0;
       while (cls + 1 < kNumClasses && m > c.class_cap[cls]) cls++;
       for (int q = 0; q < kNumClasses; q++) {
-        const bool mine = to_small && cls == (uint32_t)q;
+        const bool mine = to_small && !to_clus && cls == (uint32_t)q;
         if (!__any_sync(kFull, mine)) continue;
         const uint32_t i = warp_append(&c.cnt->small_count[q], mine ? 1u : 0u);
         if (mine) {
@@ -1682,6 +1701,128 @@ __global__ void __launch_bounds__(kSmallMaxThreads, 1)
     if constexpr (kHasVal<Val>)
       for (uint32_t q = threadIdx.x; q < m; q += nt) c.vout[I.lo + q] = sv[phys(q)];
     if (nt == 32) __syncwarp(); else __syncthreads();
+  }
+}
+
+// ---------------------------------------------------------------------------
+// Cluster-wide bucket sort (GSS_FLAG_CLUSTER_SORT): buckets
+// larger than one CTA's shared memory -- the range where the paper falls
+// back to a global-memory quicksort before its M = 2^17 --
+// are sorted by a cluster of kClusterCtas CTAs (one per SM) through
+// distributed shared memory.  CTA r loads slice [s_r, s_r+1) of the bucket
+// (s_r = floor(r m / CL)), sorts it with CtaSort, then log2(CL) merge rounds
+// pair ever larger groups of slices: each CTA produces the output positions of
+// its own slice by a merge-path search and a sequential merge whose operands
+// are read from the other CTAs' shared memory (ld through
+// cluster.map_shared_rank), into its second buffer; a cluster barrier
+// separates the rounds.  Ties take A first; the sort stays unstable.
+// ---------------------------------------------------------------------------
+constexpr int kClusterCtas = 8;
+constexpr int kClusterThreads = 512;
+template <class Key, class Val>
+constexpr uint32_t cluster_slice() { return (uint32_t)kClusterThreads * (uint32_t)small_items<Key, Val>(); }
+template <class Key, class Val>
+constexpr uint32_t cluster_capacity() { return (uint32_t)kClusterCtas * cluster_slice<Key, Val>(); }
+template <class Key, class Val>
+constexpr size_t cluster_smem_bytes() {
+  return 2 * (size_t)padded_len((int)cluster_slice<Key, Val>()) * (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0)) + 256;
+}
+
+template <class Key, class Val, class IdT, class Cmp>
+__global__ void __cluster_dims__(kClusterCtas, 1, 1) __launch_bounds__(kClusterThreads, 1)
+    k_small_cluster(Ctx<Key, Val, IdT> c) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  namespace cg = cooperative_groups;
+  cg::cluster_group cl = cg::this_cluster();
+  constexpr int CL = kClusterCtas;
+  constexpr int ITEMS = small_items<Key, Val>();
+  constexpr uint32_t C = cluster_slice<Key, Val>();
+  constexpr int PL = padded_len((int)C);
+  using Sorter = CtaSort<Key, Val, kClusterThreads, Cmp, ITEMS>;
+  const Cmp less;
+  const uint32_t r = cl.block_rank();
+  Key* kb[2];
+  Val* vb[2];
+  kb[0] = reinterpret_cast<Key*>(smem_raw);
+  kb[1] = kb[0] + PL;
+  vb[0] = reinterpret_cast<Val*>(smem_raw + 2 * (size_t)PL * sizeof(Key));
+  vb[1] = vb[0] + (kHasVal<Val> ? PL : 0);
+  uint32_t* s_sl = reinterpret_cast<uint32_t*>(smem_raw + cluster_smem_bytes<Key, Val>() - 256);   // CL+1 slice starts
+  const uint32_t ni = min(c.cnt->clus_count, c.cap_clus);
+  const uint32_t ncl = gridDim.x / CL;
+  for (uint32_t i = blockIdx.x / CL; i < ni; i += ncl) {
+    const Item I = c.clus[i];
+    const uint32_t m = I.m;
+    if (threadIdx.x <= (uint32_t)CL) s_sl[threadIdx.x] = (uint32_t)(((uint64_t)threadIdx.x * m) / CL);
+    __syncthreads();
+    const uint32_t s0 = s_sl[r], len = s_sl[r + 1] - s0;
+    const Key* src = c.keys(I.buf) + I.lo;
+    const Val* vsrc = nullptr;
+    if constexpr (kHasVal<Val>) vsrc = c.vals(I.buf) + I.lo;
+    for (uint32_t q = threadIdx.x; q < len; q += kClusterThreads) {
+      kb[0][phys(q)] = src[s0 + q];
+      if constexpr (kHasVal<Val>) vb[0][phys(q)] = vsrc[s0 + q];
+    }
+    Sorter::sort(kb[0], vb[0], (int)len, less);                    // the CTA's slice, ascending
+    cl.sync();                                                      // every slice sorted
+    uint32_t cur = 0;
+    // the bucket position pos lives in CTA owner(pos) at local slot pos - s_owner
+    auto owner = [&](uint32_t pos) -> uint32_t {
+      uint32_t o = (uint32_t)(((uint64_t)CL * (pos + 1) + m - 1) / m) - 1;
+      return min(o, (uint32_t)CL - 1);
+    };
+    auto ldk = [&](uint32_t pos) -> Key {
+      const uint32_t o = owner(pos);
+      const Key* rk = cl.map_shared_rank(kb[cur], o);
+      return rk[phys(pos - s_sl[o])];
+    };
+    auto ldv = [&](uint32_t pos) -> Val {
+      const uint32_t o = owner(pos);
+      const Val* rv = cl.map_shared_rank(vb[cur], o);
+      return rv[phys(pos - s_sl[o])];
+    };
+    for (int w = 1; w < CL; w *= 2) {
+      const uint32_t g = r / (2 * w);
+      const uint32_t a0 = s_sl[g * 2 * w], b0 = s_sl[min(g * 2 * w + w, (uint32_t)CL)];
+      const uint32_t b1 = s_sl[min(g * 2 * w + 2 * w, (uint32_t)CL)];
+      const uint32_t aLen = b0 - a0, bLen = b1 - b0;
+      Key* ok = kb[cur ^ 1];
+      Val* ov = vb[cur ^ 1];
+      for (uint32_t o0 = threadIdx.x * ITEMS; o0 < len; o0 += kClusterThreads * ITEMS) {
+        const uint32_t cnt = min((uint32_t)ITEMS, len - o0);
+        const uint32_t d = s0 - a0 + o0;                            // output diagonal inside the pair
+        // j = number of A keys among the first d outputs (A first on ties):
+        // the smallest j in [lo, hi) with B[d-1-j] < A[j], else hi
+        uint32_t lo = d > bLen ? d - bLen : 0, hi = min(d, aLen);
+        while (lo < hi) {
+          const uint32_t mid = (lo + hi) >> 1;
+          if (less(ldk(b0 + d - 1 - mid), ldk(a0 + mid))) hi = mid;
+          else lo = mid + 1;
+        }
+        uint32_t xa = lo, xb = d - lo;
+        Key ka{}, kbk{};
+        Val va{}, vbv{};
+        if (xa < aLen) { ka = ldk(a0 + xa); if constexpr (kHasVal<Val>) va = ldv(a0 + xa); }
+        if (xb < bLen) { kbk = ldk(b0 + xb); if constexpr (kHasVal<Val>) vbv = ldv(b0 + xb); }
+        for (uint32_t j = 0; j < cnt; j++) {
+          const bool ta = xb >= bLen || (xa < aLen && !less(kbk, ka));
+          ok[phys(o0 + j)] = ta ? ka : kbk;
+          if constexpr (kHasVal<Val>) ov[phys(o0 + j)] = ta ? va : vbv;
+          if (ta) {
+            if (++xa < aLen) { ka = ldk(a0 + xa); if constexpr (kHasVal<Val>) va = ldv(a0 + xa); }
+          } else {
+            if (++xb < bLen) { kbk = ldk(b0 + xb); if constexpr (kHasVal<Val>) vbv = ldv(b0 + xb); }
+          }
+        }
+      }
+      cl.sync();                                                    // every read of this round's input is done
+      cur ^= 1;
+    }
+    for (uint32_t q = threadIdx.x; q < len; q += kClusterThreads) {
+      c.kout[I.lo + s0 + q] = kb[cur][phys(q)];
+      if constexpr (kHasVal<Val>) c.vout[I.lo + s0 + q] = vb[cur][phys(q)];
+    }
+    cl.sync();                                                      // buffers free for the next bucket
   }
 }
 

@@ -645,3 +645,44 @@ def test_ablation_variants_vs_oracle(gss, oracle_mod, width, pairs, variant):
         check_pairs(x, to_host(vo), ok)
     if st is not None:
         assert_levels_match(st, recs)
+
+
+# ---------------------------------------------------------------------------
+# Cluster-wide bucket sort (GSS_FLAG_CLUSTER_SORT = 256):
+# buckets between one CTA's and a cluster's capacity, against the oracle
+# ---------------------------------------------------------------------------
+CLUSTER_CAP = {(32, False): 8 * 512 * 32, (64, False): 8 * 512 * 16, (32, True): 8 * 512 * 16,
+               (64, True): 8 * 512 * 8}
+CTA_CAP = {(32, False): 32768, (64, False): 16384, (32, True): 16384, (64, True): 8192}
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("dist", ["uniform", "and4", "sorted"])
+def test_cluster_sort_vs_oracle(gss, oracle_mod, width, pairs, dist):
+    M = CLUSTER_CAP[(width, pairs)]
+    n = 48 * (M // 2) + 555                          # level 0 at k = 64 leaves buckets of ~0.75 M > one CTA
+    x = inputs.keys(dist, n, width, seed=41)
+    v = inputs.values(n, width) if pairs else None
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, k=64, M=M, k_policy="fixed"), log=True)
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, k=64, k_policy="fixed", M=M, flags=256,
+                          stats=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if pairs:
+        check_pairs(x, to_host(vo), ok)
+    assert_levels_match(st, recs)
+    if dist != "and4":
+        assert st.cluster_buckets > 0 and st.max_small > CTA_CAP[(width, pairs)]
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+def test_cluster_sort_single_bucket(gss, width, pairs):
+    """n <= M: the whole input is one bucket for one cluster (sizes around the slice boundaries)."""
+    cap = CLUSTER_CAP[(width, pairs)]
+    for n in (CTA_CAP[(width, pairs)] + 1, cap // 2 + 3, cap - 1, cap):
+        x = inputs.keys("uniform", n, width, seed=n)
+        v = inputs.values(n, width) if pairs else None
+        ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, flags=256, stats=True)
+        np.testing.assert_array_equal(to_host(ko), np.sort(x), err_msg=f"n={n}")
+        if pairs:
+            check_pairs(x, to_host(vo), np.sort(x))
+        assert st.cluster_buckets == 1 and st.levels == 0
