@@ -207,6 +207,23 @@ __device__ __forceinline__ Key ld_shared(uint32_t a) {
     return bit_cast_dev<Key>(x);
   }
 }
+// Two adjacent keys (a 2W-byte aligned pair) by one shared load.
+template <class Key>
+__device__ __forceinline__ void ld_shared_pair(uint32_t a, Key& x0, Key& x1) {
+  if constexpr (sizeof(Key) == 8) {
+    unsigned long long u0, u1;
+    asm volatile("ld.shared.v2.u64 {%0, %1}, [%2];" : "=l"(u0), "=l"(u1) : "r"(a));
+    x0 = bit_cast_dev<Key>(u0); x1 = bit_cast_dev<Key>(u1);
+  } else {
+    uint32_t u0, u1;
+    asm volatile("ld.shared.v2.u32 {%0, %1}, [%2];" : "=r"(u0), "=r"(u1) : "r"(a));
+    x0 = bit_cast_dev<Key>(u0); x1 = bit_cast_dev<Key>(u1);
+  }
+}
+#ifndef GSS_CLS_PAIRLOAD
+#define GSS_CLS_PAIRLOAD 0
+#endif
+
 __device__ __forceinline__ void red_shared_add(uint32_t a, uint32_t v) {
   asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(a), "r"(v));
 }
@@ -256,7 +273,23 @@ __device__ __forceinline__ void descend_group(const Key (&e)[U], uint32_t (&id)[
   uint32_t r[U];
 #pragma unroll
   for (int u = 0; u < U; u++) r[u] = W;
-  for (uint32_t d = 0; d < d1; d++) {
+  uint32_t d = 0;
+#if GSS_CLS_PAIRLOAD
+  // two levels per round trip: node j and both children (2j, 2j+1 are adjacent: one 2W-byte load)
+  // are loaded together, so the dependent chain has one shared-memory latency per two levels
+  for (; d + 2 <= d1; d += 2) {
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const Key x = ld_shared<Key>(tree_s + r[u]);
+      Key c0, c1;
+      ld_shared_pair<Key>(tree_s + 2 * r[u], c0, c1);
+      const bool p1 = less(x, e[u]);
+      const bool p2 = less(p1 ? c1 : c0, e[u]);
+      r[u] = 4 * r[u] + (p1 ? 2 * W : 0u) + (p2 ? W : 0u);
+    }
+  }
+#endif
+  for (; d < d1; d++) {
 #pragma unroll
     for (int u = 0; u < U; u++) {
       const Key x = ld_shared<Key>(tree_s + r[u]);
@@ -952,6 +985,10 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   constexpr int NW = kScatterThreads / 32;
   using SM = ScatterBulkSmem<Key, Val, IdT>;
   constexpr uint32_t A = SM::A;
+  // keys only: one counter set per CTA (ranks in the hardware's atomic order across warps; equal keys are
+  // bit-identical, so the output stays deterministic) -- no per-warp fold.  With values: per-warp counters,
+  // whose fixed fold order keeps the values of equal keys deterministic.
+  constexpr bool CTA_CNT = !kHasVal<Val>;
   uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);       // next global index of each id (this tile)
   uint32_t* rstart = gbase + kmax;                                // staging slot of each id's run (this chunk)
   uint32_t* rlen = rstart + kmax;                                 // run length of each id (this chunk)
@@ -971,7 +1008,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   if constexpr (kHasVal<Val>) { vsrc = c.vals(sb); vdst = c.wvals(db); }
   const IdT* idsrc = c.ids;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  uint32_t* wc = wcnt + w * kmax;
+  uint32_t* wc = CTA_CNT ? wcnt : wcnt + w * kmax;
   const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
   const uint32_t q0 = w * (32 * kScatterIter) + lane;
 
@@ -1018,6 +1055,10 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   };
   uint32_t c0 = 0, buf = 0;
   load_chunk(beg, idb, min((uint32_t)kChunk, len));
+  if constexpr (CTA_CNT) {
+    for (uint32_t id = threadIdx.x; id < kmax; id += kScatterThreads) wcnt[id] = 0;
+    __syncthreads();
+  }
   for (;;) {
     Key kk[kScatterIter];
     Val vv[kScatterIter];
@@ -1029,8 +1070,10 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       if constexpr (kHasVal<Val>) vv[it] = pv[it];
     }
     const uint32_t cur_K = K;
-    for (uint32_t id = lane; id < cur_K; id += 32) wc[id] = 0;
-    __syncwarp();
+    if constexpr (!CTA_CNT) {
+      for (uint32_t id = lane; id < cur_K; id += 32) wc[id] = 0;
+      __syncwarp();
+    }
     // ranks within (warp, id): one shared atomic per key on the warp's own counters
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
@@ -1046,8 +1089,13 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       const uint32_t id = i0 + j;
       if (id < cur_K) {
         uint32_t tt = 0;
+        if constexpr (CTA_CNT) {
+          tt = wcnt[id];
+          wcnt[id] = 0;                                           // reset for the next chunk (its atomics follow B3)
+        } else {
 #pragma unroll
-        for (int q = 0; q < NW; q++) tt += wcnt[q * kmax + id];
+          for (int q = 0; q < NW; q++) tt += wcnt[q * kmax + id];
+        }
         rlen[id] = tt;
         tsum += tt + (A - 1);
       }
@@ -1064,12 +1112,14 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
         }
         const uint32_t st = ex + ((dal - ex) & (A - 1));            // staging slot == destination (mod A)
         rstart[id] = st;
-        uint32_t run = st;
+        if constexpr (!CTA_CNT) {
+          uint32_t run = st;
 #pragma unroll
-        for (int q = 0; q < NW; q++) {
-          const uint32_t x = wcnt[q * kmax + id];
-          wcnt[q * kmax + id] = run;
-          run += x;
+          for (int q = 0; q < NW; q++) {
+            const uint32_t x = wcnt[q * kmax + id];
+            wcnt[q * kmax + id] = run;
+            run += x;
+          }
         }
         ex += L + (A - 1);
       }
@@ -1081,7 +1131,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
 #pragma unroll
     for (int it = 0; it < kScatterIter; it++) {
       if (iid[it] != 0xffffffffu) {
-        const uint32_t pos = wc[iid[it] & 0xffffu] + (iid[it] >> 16);
+        const uint32_t pos = (CTA_CNT ? rstart[iid[it] & 0xffffu] : wc[iid[it] & 0xffffu]) + (iid[it] >> 16);
         sk[pos] = kk[it];
         if constexpr (kHasVal<Val>) sv[pos] = vv[it];
       }
