@@ -366,6 +366,10 @@ struct Engine {
     using SBS = ScatterBulkSmem<Key, Val, IdT>;
     const bool bulk2 = SBS::bytes(kmax, 2) <= 113 * 1024;
     auto ksb = bulk2 ? k_scatter_bulk<Key, Val, IdT, 2> : k_scatter_bulk<Key, Val, IdT, 1>;
+    if constexpr (!kHasVal<Val>) {
+      if (cfg.flags & kFlagScatterCtaCounters)   // ablation: one counter set per CTA (nondeterministic intermediates)
+        ksb = bulk2 ? k_scatter_bulk<Key, Val, IdT, 2, true> : k_scatter_bulk<Key, Val, IdT, 1, true>;
+    }
     const size_t sm_sb = SBS::bytes(kmax, bulk2 ? 2 : 1);
     GSS_TRY(set_smem(ksb, sm_sb));
     const int g_sb = grid_for(ksb, kScatterThreads, sm_sb, di.sms);
@@ -373,7 +377,8 @@ struct Engine {
     // for 4-byte keys the per-run copies (one warp-serialised UBLKCP each) cost more than the
     // coalesced per-key stores they replace (2^27 u32: 1.26 vs 1.05 ms), so those keep GSS_FLAG_SCATTER_REGS
     const bool use_bulk = c.nremote || (!c.stable && !c.recompute && (sizeof(Key) == 8 || (cfg.flags & kFlagScatterBulk)) &&
-                          !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters | GSS_FLAG_SCATTER_REGS)));
+                          !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS)) &&
+                          !((cfg.flags & kFlagScatterCtaCounters) && kHasVal<Val>));
     auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
     const size_t sm_sd = (size_t)kmax * 4;
     GSS_TRY(set_smem(ksd, sm_sd));

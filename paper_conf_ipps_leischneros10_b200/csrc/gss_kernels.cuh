@@ -976,7 +976,7 @@ struct ScatterBulkSmem {
   static size_t bytes(uint32_t kmax, int nbuf) { return head_bytes(kmax) + (size_t)nbuf * (key_bytes(kmax) + val_bytes(kmax)); }
 };
 
-template <class Key, class Val, class IdT, int NBUF>
+template <class Key, class Val, class IdT, int NBUF, bool CTA_CNT = false>
 __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     k_scatter_bulk(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
@@ -985,10 +985,11 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   constexpr int NW = kScatterThreads / 32;
   using SM = ScatterBulkSmem<Key, Val, IdT>;
   constexpr uint32_t A = SM::A;
-  // keys only: one counter set per CTA (ranks in the hardware's atomic order across warps; equal keys are
-  // bit-identical, so the output stays deterministic) -- no per-warp fold.  With values: per-warp counters,
-  // whose fixed fold order keeps the values of equal keys deterministic.
-  constexpr bool CTA_CNT = !kHasVal<Val>;
+  // CTA_CNT (ablation, keys only): one counter set per CTA -- no per-warp fold (2^28 u64: 2.75 vs 2.92 ms for
+  // the two levels), but ranks follow the hardware's atomic order across warps, so the order of keys inside a
+  // bucket, hence the next level's sample and splitters, vary from run to run (final keys do not).  Default:
+  // per-warp counters folded in a fixed order, deterministic intermediates that match the oracle's level
+  // records.
   uint32_t* gbase = reinterpret_cast<uint32_t*>(smem_raw);       // next global index of each id (this tile)
   uint32_t* rstart = gbase + kmax;                                // staging slot of each id's run (this chunk)
   uint32_t* rlen = rstart + kmax;                                 // run length of each id (this chunk)
