@@ -37,6 +37,7 @@ namespace gssh {
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
 inline constexpr uint32_t kFlagScatterBulk = 1u << 29;          // ablation: bulk-copy scatter for 4-byte keys too
+inline constexpr uint32_t kFlagSmallWide = 1u << 28;            // ablation: one 64-register block sort for every class
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -323,13 +324,19 @@ struct Engine {
       return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, ns, smem, s>>>(c, (uint32_t)cls); });
     }
     auto kern = k_small_block<Key, Val, IdT, Cmp>;
+    // register-capped instantiation for the narrower classes (not for 4-byte keys with values: it spills)
+    constexpr bool kNarrowOk = !(kHasVal<Val> && sizeof(Key) == 4);
+    const bool narrow = kNarrowOk && nt <= kSmallNarrowThreads && !(cfg.flags & kFlagSmallWide);
+    if constexpr (kNarrowOk) {
+      if (narrow) kern = k_small_block<Key, Val, IdT, Cmp, false, kSmallNarrowThreads>;
+    }
     if constexpr (sizeof(Key) == 8 && !kHasVal<Val> && std::is_same<Cmp, Less>::value) {
       if (cfg.flags & GSS_FLAG_BITONIC_NET) kern = k_small_block<Key, Val, IdT, Cmp, true>;   // ablation
     }
     const size_t smem = block_sort_smem_bytes<Key, Val>(nt);
-    GSS_TRY(set_smem(kern, block_sort_smem_bytes<Key, Val>(kSmallMaxThreads)));
-    static GridCache grid[2][kNumClasses + 1];
-    const int gv = (cfg.flags & GSS_FLAG_BITONIC_NET) ? 1 : 0;
+    GSS_TRY(set_smem(kern, block_sort_smem_bytes<Key, Val>(narrow ? kSmallNarrowThreads : kSmallMaxThreads)));
+    static GridCache grid[4][kNumClasses + 1];
+    const int gv = ((cfg.flags & GSS_FLAG_BITONIC_NET) ? 1 : 0) + (narrow ? 2 : 0);
     int g = grid[gv][cls].get(di.dev);
     if (!g) { g = grid_for(kern, nt, smem, di.sms); grid[gv][cls].put(di.dev, g); }
     return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, nt, smem, s>>>(c, (uint32_t)cls); });

@@ -15,6 +15,6 @@ for spec in "k_classify:k_classify:1" "k_scatter:k_scatter:1" "k_small:k_small_b
      > gpurun_out/prof_${TAG}_${N}.log 2>&1
   echo "$N rc=$?"
 done
-cp paper_conf_ipps_leischneros10_b200/libgss.so gpurun_out/libgss_${TAG}.so
+# (the profiled libgss.so stays on the box: gpurun_out/ must stay under 64 MiB; rebuild the commit to map SASS lines)
 python tools/summarize_profiles.py $TAG $WL paper_conf_ipps_leischneros10_b200/libgss.so gpurun_out > gpurun_out/summarize_${TAG}.log 2>&1
 echo "summary rc=$?"
