@@ -107,6 +107,10 @@ typedef struct gss_params {
                                arrays; ablation SURVEY NEXT-4 iii)               */
   gss_stats* stats;         /* optional host pointer: the call syncs and fills it          */
   gss_profiler* profiler;   /* optional: CUDA-event time of every launch                   */
+  uint32_t* error_out;      /* optional DEVICE pointer: a sort copies its internal
+                               capacity-check flags there, stream ordered, without a host
+                               sync (0 = the result is valid; also captured by
+                               GSS_FLAG_GRAPH)                                              */
 } gss_params;
 
 #define GSS_FLAG_RECOMPUTE_IDS 1u  /* Phase 4 re-descends the splitter tree instead of reading

@@ -39,7 +39,7 @@ class _Stats(ctypes.Structure):
 class _Params(ctypes.Structure):
     _fields_ = [("k", _u32), ("oversample", _u32), ("small_threshold", _u64), ("tile", _u32),
                 ("max_levels", _u32), ("k_policy", _u32), ("fill_div", _u32), ("seed", _u64), ("flags", _u32),
-                ("cls_arrays", _u32), ("stats", ctypes.POINTER(_Stats)), ("profiler", _vp)]
+                ("cls_arrays", _u32), ("stats", ctypes.POINTER(_Stats)), ("profiler", _vp), ("error_out", _vp)]
 
 
 @dataclass
@@ -166,7 +166,7 @@ class Profiler:
 
 
 def _params(k=None, M=None, a=None, tile=None, seed=None, k_policy=None, fill_div=None, max_levels=None,
-            flags=0, stats=None, profiler=None, cls_arrays=None):
+            flags=0, stats=None, profiler=None, cls_arrays=None, error_out=None):
     p = _Params()
     p.k = k or 0
     p.small_threshold = M or 0
@@ -178,6 +178,10 @@ def _params(k=None, M=None, a=None, tile=None, seed=None, k_policy=None, fill_di
     p.max_levels = max_levels or 0
     p.flags = flags
     p.cls_arrays = cls_arrays or 0
+    if error_out is not None:
+        if not (error_out.is_cuda and error_out.dtype in (torch.int32, torch.uint32) and error_out.numel() >= 1):
+            raise ValueError("error_out must be a CUDA int32/uint32 tensor")
+        p.error_out = error_out.data_ptr()
     if stats is not None:
         p.stats = ctypes.pointer(stats)
     if profiler is not None:

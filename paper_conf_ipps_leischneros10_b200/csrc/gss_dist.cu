@@ -210,7 +210,7 @@ inline bool fused_mode(const gss_params* p) { return p && (p->flags & GSS_FLAG_D
 inline gss_params sub_params(const gss_params* p, bool keep_stats) {
   gss_params q{};
   if (p) q = *p;
-  if (!keep_stats) q.stats = nullptr;
+  if (!keep_stats) { q.stats = nullptr; q.error_out = nullptr; }
   q.flags &= ~GSS_FLAG_GRAPH;   // the buffers of the sub-calls change with the received count
   return q;
 }

@@ -72,6 +72,7 @@ inline gss_status device_info(DeviceInfo* out) {
 struct Cfg {
   uint32_t k, a, T, L, k_policy, fill_div, flags, kmax, nclass, cls_arrays;
   uint64_t M, seed;
+  uint32_t* error_out;
   uint32_t class_cap[kNumClasses];
 };
 
@@ -113,6 +114,7 @@ gss_status resolve(const gss_params* up, uint64_t n, Cfg* c, uint32_t kmin_given
   c->fill_div = p.fill_div ? p.fill_div : 4;
   c->seed = p.seed ? p.seed : 5489;
   c->flags = p.flags;
+  c->error_out = p.error_out;
   c->cls_arrays = p.cls_arrays ? p.cls_arrays : 8;
   if (c->cls_arrays != 1 && c->cls_arrays != 2 && c->cls_arrays != 4 && c->cls_arrays != 8) return GSS_ERROR_INVALID_VALUE;
   // size classes (R8): class i = buckets a CTA of class_warps(i) warps sorts
@@ -438,6 +440,13 @@ struct Engine {
     const size_t sm_ovf = CtaSort<Key, Val, NTO, Cmp>::smem_bytes();
     GSS_TRY(set_smem(ko, sm_ovf));
     GSS_TRY(launch(prof, GSS_K_OVERFLOW, s, count, [&] { ko<<<di.sms, NTO, sm_ovf, s>>>(c); }));
+    if (cfg.error_out) {
+      // the capacity-check flags of this sort (0 = the result is valid), stream ordered, no host sync
+      if (cudaMemcpyAsync(cfg.error_out, &c.cnt->err, sizeof(uint32_t), cudaMemcpyDeviceToDevice, s) != cudaSuccess) {
+        cudaGetLastError();
+        return GSS_ERROR_CUDA;
+      }
+    }
     return GSS_SUCCESS;
   }
 };
@@ -468,7 +477,7 @@ struct GraphKey {
   const void* fn;
   int dev;
   uint64_t n;
-  const void* p[5];
+  const void* p[6];
   uint32_t cfg[8];
   uint64_t seed;
   bool operator==(const GraphKey& o) const { return memcmp(this, &o, sizeof(GraphKey)) == 0; }
@@ -619,6 +628,7 @@ gss_status drive(IO io, size_t n, void* temp, size_t* temp_bytes, void* stream, 
       key.dev = di.dev;
       key.n = n;
       key.p[0] = io.kin; key.p[1] = io.kout; key.p[2] = io.vin; key.p[3] = io.vout; key.p[4] = temp;
+      key.p[5] = cfg.error_out;
       key.cfg[0] = cfg.k; key.cfg[1] = cfg.a; key.cfg[2] = cfg.T; key.cfg[3] = cfg.L; key.cfg[4] = cfg.k_policy;
       key.cfg[5] = cfg.fill_div | (cfg.cls_arrays << 24); key.cfg[6] = cfg.flags; key.cfg[7] = (uint32_t)cfg.M;
       key.seed = cfg.seed;

@@ -686,3 +686,22 @@ def test_cluster_sort_single_bucket(gss, width, pairs):
         if pairs:
             check_pairs(x, to_host(vo), np.sort(x))
         assert st.cluster_buckets == 1 and st.levels == 0
+
+
+
+def test_error_out_flags(gss):
+    """gss_params.error_out: the capacity-check flags land in a device word without a host sync,
+    on the direct path and through the CUDA-graph replay; 0 for a valid result."""
+    n = (1 << 20) + 5
+    x = inputs.keys("and2", n, 64, seed=8)
+    err = torch.full((1,), 0x7fffffff, dtype=torch.int32, device="cuda")
+    ko, _ = gss.sort(to_dev(x), error_out=err)
+    assert int(err.item()) == 0
+    np.testing.assert_array_equal(to_host(ko), np.sort(x))
+    s = gss.Sorter("u64", n, False, flags=16, error_out=err)
+    kin, kout = to_dev(x), torch.empty(n, dtype=torch.uint64, device="cuda")
+    for _ in range(2):
+        err.fill_(0x7fffffff)
+        s(kin, kout)
+        assert int(err.item()) == 0
+    np.testing.assert_array_equal(to_host(kout), np.sort(x))
