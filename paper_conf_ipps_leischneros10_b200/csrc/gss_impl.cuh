@@ -37,7 +37,8 @@ namespace gssh {
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
 inline constexpr uint32_t kFlagScatterBulk = 1u << 29;          // ablation: bulk-copy scatter for 4-byte keys too
-inline constexpr uint32_t kFlagSmallWide = 1u << 28;            // ablation: one 64-register block sort for every class
+inline constexpr uint32_t kFlagSmallNarrow = 1u << 28;          // ablation: 48-register block sort for classes <= 20 warps
+                                                                // (2^28 u64: 4.98 vs 4.90 ms -- occupancy is not the limit)
 
 inline size_t align_up(size_t x, size_t a = 256) { return (x + a - 1) / a * a; }
 
@@ -326,9 +327,9 @@ struct Engine {
       return launch(prof, GSS_K_SMALL_SORT, s, count, [&] { kern<<<g, ns, smem, s>>>(c, (uint32_t)cls); });
     }
     auto kern = k_small_block<Key, Val, IdT, Cmp>;
-    // register-capped instantiation for the narrower classes (not for 4-byte keys with values: it spills)
+    // ablation: register-capped instantiation for the narrower classes (not for 4-byte keys with values: it spills)
     constexpr bool kNarrowOk = !(kHasVal<Val> && sizeof(Key) == 4);
-    const bool narrow = kNarrowOk && nt <= kSmallNarrowThreads && !(cfg.flags & kFlagSmallWide);
+    const bool narrow = kNarrowOk && nt <= kSmallNarrowThreads && (cfg.flags & kFlagSmallNarrow);
     if constexpr (kNarrowOk) {
       if (narrow) kern = k_small_block<Key, Val, IdT, Cmp, false, kSmallNarrowThreads>;
     }

@@ -1693,8 +1693,9 @@ __host__ __device__ constexpr size_t block_sort_smem_bytes(int nt) {
 #ifndef GSS_SMALL_CPASYNC
 #define GSS_SMALL_CPASYNC 1   // 8-byte keys: 4.83 vs 4.96 ms (2^28 u64), pairs 4.45 vs 4.57; 4-byte copies lose (2.15 vs 1.58)
 #endif
-// MAXT: the widest CTA the instantiation serves.  Classes of up to 20 warps use MAXT = 640 with two
-// resident CTAs guaranteed, which caps the registers at 48 (from 60): four 10-warp CTAs per SM instead of three.
+// MAXT: the widest CTA the instantiation serves.  The ablation kFlagSmallNarrow gives classes of up to 20
+// warps MAXT = 640 with two resident CTAs guaranteed, which caps the registers at 48 (from 60): four 10-warp
+// CTAs per SM instead of three -- measured no faster (2^28 u64 4.98 vs 4.90 ms).
 constexpr int kSmallNarrowThreads = 640;
 template <class Key, class Val, class IdT, class Cmp, bool BITONIC = false, int MAXT = kSmallMaxThreads>
 __global__ void __launch_bounds__(MAXT, MAXT <= kSmallNarrowThreads ? 2 : 1)
