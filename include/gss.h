@@ -127,10 +127,10 @@ typedef struct gss_params {
                                       CUDA graph on first use and replay it on later calls
                                       with identical buffers, n and parameters (launch-bound
                                       sizes); ignored with stats or a profiler              */
-#define GSS_FLAG_SCATTER_REGS 32u  /* 8-byte keys: Phase 4 writes bucket runs with per-key
-                                      shared loads and coalesced global stores (the round-1
-                                      scatter; ablation) instead of one bulk copy
-                                      (cp.async.bulk) per run; 4-byte keys always do         */
+#define GSS_FLAG_SCATTER_REGS 32u  /* 8-byte keys without values: Phase 4 writes bucket runs
+                                      with per-key shared loads and coalesced global stores
+                                      (the round-1 scatter; ablation) instead of one bulk copy
+                                      (cp.async.bulk) per run; every other kind always does  */
 #define GSS_FLAG_DIST_FUSED 64u    /* gss_dist_sort_*: fuse the global scatter with the exchange
                                       (SURVEY NEXT-1): the partition's bucket runs are stored
                                       by the scatter kernel straight into the receiving GPU's

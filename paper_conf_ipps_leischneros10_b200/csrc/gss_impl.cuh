@@ -383,10 +383,12 @@ struct Engine {
     const size_t sm_sb = SBS::bytes(kmax, bulk2 ? 2 : 1);
     GSS_TRY(set_smem(ksb, sm_sb));
     const int g_sb = grid_for(ksb, kScatterThreads, sm_sb, di.sms);
-    // bulk copies pay for 8-byte keys (2^28 u64: 2.90 vs 3.11 ms for the two levels; u64 pairs equal);
-    // for 4-byte keys the per-run copies (one warp-serialised UBLKCP each) cost more than the
-    // coalesced per-key stores they replace (2^27 u32: 1.26 vs 1.05 ms), so those keep GSS_FLAG_SCATTER_REGS
-    const bool use_bulk = c.nremote || (!c.stable && !c.recompute && (sizeof(Key) == 8 || (cfg.flags & kFlagScatterBulk)) &&
+    // bulk copies pay for 8-byte keys alone (2^28 u64: 2.92 vs 3.11 ms for the two levels); with values
+    // they do not (2^27 u64 pairs 3.02 vs 2.99 ms; 2^29 pairs, k = 512, one staging buffer: 18.0 vs 16.8 ms),
+    // nor for 4-byte keys, where the per-run copies (one warp-serialised UBLKCP each) cost more than the
+    // coalesced per-key stores they replace (2^27 u32: 1.26 vs 1.05 ms); those keep GSS_FLAG_SCATTER_REGS
+    const bool bulk_default = sizeof(Key) == 8 && !kHasVal<Val>;
+    const bool use_bulk = c.nremote || (!c.stable && !c.recompute && (bulk_default || (cfg.flags & kFlagScatterBulk)) &&
                           !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS)) &&
                           !((cfg.flags & kFlagScatterCtaCounters) && kHasVal<Val>));
     auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
