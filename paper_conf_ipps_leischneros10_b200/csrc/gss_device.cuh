@@ -355,6 +355,58 @@ __device__ __forceinline__ void thread_sort_net(Key* k, Val* v, Cmp less) {
   else oem_sort<0, N>(k, v, less);
 }
 
+// Bitonic merges across the 32 lanes of a warp, in registers (no shared
+// memory, no warp barrier): every lane holds ITEMS keys sorted ascending
+// (blocked: lane l has slots [l*ITEMS, (l+1)*ITEMS)); step s merges pairs of
+// sorted runs of ITEMS*2^s keys (groups of 2^s lanes) into ascending runs of
+// twice that length: a flip stage (slot g against slot L-1-g of the merged
+// group, the lower slot keeps the minimum) followed by half-cleaners with
+// strides L/4 .. 1, across lanes (shuffles) while the stride is >= ITEMS and
+// inside the lane's registers below.  After the five steps the warp's
+// 32*ITEMS keys are sorted ascending.  The paper's bitonic alternative
+// (P:339-341), applied across lanes where the odd-even merge sort's merge-path
+// rounds would cost shared-memory round trips and warp barriers.
+template <int ITEMS, class Key, class Cmp>
+__device__ __forceinline__ void warp_bitonic_merges(Key (&k)[ITEMS], int lane, Cmp less) {
+#pragma unroll
+  for (int s = 0; s < 5; s++) {
+    const int gmask = (2 << s) - 1;
+    const bool lower = (lane & (1 << s)) == 0;
+#pragma unroll
+    for (int i = 0; i < ITEMS / 2; i++) {
+      const int j = ITEMS - 1 - i;
+      const Key yi = __shfl_xor_sync(kFull, k[j], gmask);      // partner slot ITEMS-1-i for my slot i
+      const Key yj = __shfl_xor_sync(kFull, k[i], gmask);      // partner slot i for my slot j
+      const bool ti = lower ? less(yi, k[i]) : less(k[i], yi);
+      const bool tj = lower ? less(yj, k[j]) : less(k[j], yj);
+      k[i] = ti ? yi : k[i];
+      k[j] = tj ? yj : k[j];
+    }
+#pragma unroll
+    for (int dl = (1 << s) >> 1; dl >= 1; dl >>= 1) {
+      const bool lo = (lane & dl) == 0;
+#pragma unroll
+      for (int i = 0; i < ITEMS; i++) {
+        const Key y = __shfl_xor_sync(kFull, k[i], dl);
+        const bool t = lo ? less(y, k[i]) : less(k[i], y);
+        k[i] = t ? y : k[i];
+      }
+    }
+#pragma unroll
+    for (int d = ITEMS / 2; d >= 1; d >>= 1) {
+#pragma unroll
+      for (int i = 0; i < ITEMS; i++) {
+        if ((i & d) == 0) {
+          const bool sw = less(k[i + d], k[i]);
+          const Key a = sw ? k[i + d] : k[i], b = sw ? k[i] : k[i + d];
+          k[i] = a;
+          k[i + d] = b;
+        }
+      }
+    }
+  }
+}
+
 // Stable odd-even transposition sort (only for the one partial thread).
 template <int N, class Key, class Val, class Cmp>
 __device__ __forceinline__ void transposition_sort(Key* k, Val* v, Cmp less) {
@@ -655,6 +707,14 @@ struct CtaSort {
   // thread of the nt-thread block (nt <= NT; nt = NT unless the caller sizes
   // the block at run time), or every lane of the warp when NT == 32, must
   // call it.  Begins and ends with a barrier.
+  // keys only, bit-identical equivalents: the first five merge rounds run
+  // across the warp's registers (warp_bitonic_merges) instead of through
+  // shared memory
+#ifndef GSS_WARP_BITONIC
+#define GSS_WARP_BITONIC 1
+#endif
+  static constexpr bool WB = GSS_WARP_BITONIC && !KV && BitwiseOrder<Cmp>::value && !BITONIC;
+
   __device__ static void sort(Key* sk, Val* sv, int m, Cmp less, int nt = NT) {
     bar(nt);
     const int t = NT == 32 ? (threadIdx.x & 31) : threadIdx.x;
@@ -662,7 +722,41 @@ struct CtaSort {
     const int cnt = min(max(m - base, 0), ITEMS);
     Key k[ITEMS];
     Val v[ITEMS];
-    if (cnt > 0) {
+    int w0 = ITEMS;                                      // width of the runs the merge-path rounds start from
+    if constexpr (WB) {
+      const int lane = threadIdx.x & 31;
+      const int wbase = base - lane * ITEMS;             // the warp's first slot
+      const int wcount = min(max(m - wbase, 0), 32 * ITEMS);
+      if (wcount > 0) {                                  // warp-uniform
+        bool has = cnt > 0;
+        Key mx{};
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          if (i < cnt) {
+            k[i] = sk[phys(base + i)];
+            if (i == 0 || less(mx, k[i])) mx = k[i];
+          }
+        }
+        // pads: copies of the warp's largest key (indistinguishable from it), so the warp's real keys
+        // come out as its first wcount sorted slots
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) {
+          const Key y = __shfl_xor_sync(kFull, mx, o);
+          const bool hy = __shfl_xor_sync(kFull, has, o);
+          if (hy && (!has || less(mx, y))) mx = y;
+          has = has || hy;
+        }
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++)
+          if (i >= cnt) k[i] = mx;
+        thread_sort_net<ITEMS, BITONIC>(k, v, less);
+        warp_bitonic_merges<ITEMS>(k, lane, less);
+        const int my = min(max(wcount - lane * ITEMS, 0), ITEMS);
+        __syncwarp();
+        if (my > 0) store_run(sk, sv, k, v, my, wbase, wcount, lane * ITEMS, ((wbase / (32 * ITEMS)) & 1) != 0);
+      }
+      w0 = 32 * ITEMS;
+    } else if (cnt > 0) {
 #pragma unroll
       for (int i = 0; i < ITEMS; i++) {
         if (i < cnt) {
@@ -704,11 +798,13 @@ struct CtaSort {
         thread_sort_net<ITEMS, BITONIC>(k, v, less);
       }
     }
-    __syncwarp();
-    if (cnt > 0) store_run(sk, sv, k, v, cnt, base, cnt, 0, (t & 1) != 0);   // run t: descending if t is odd
+    if constexpr (!WB) {
+      __syncwarp();
+      if (cnt > 0) store_run(sk, sv, k, v, cnt, base, cnt, 0, (t & 1) != 0);   // run t: descending if t is odd
+    }
     // Rounds whose merged pairs (2w keys) lie inside one warp's 32*ITEMS keys
     // only synchronise the warp; wider rounds synchronise the block.
-    for (int w = ITEMS; w < m; w *= 2) {
+    for (int w = w0; w < m; w *= 2) {
       const bool blk = NT > 32 && nt > 32 && 2 * w > 32 * ITEMS;
       if (blk) __syncthreads(); else __syncwarp();
       const int ps = base & ~(2 * w - 1);                // w is a power of two
