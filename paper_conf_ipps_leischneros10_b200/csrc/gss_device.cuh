@@ -711,7 +711,7 @@ struct CtaSort {
   // across the warp's registers (warp_bitonic_merges) instead of through
   // shared memory
 #ifndef GSS_WARP_BITONIC
-#define GSS_WARP_BITONIC 1
+#define GSS_WARP_BITONIC 0   // 1: measured 2x slower (2^28 u64 in-SM sort 8.35 vs 4.91 ms; 2^27 u32 3.24 vs 1.61)
 #endif
   static constexpr bool WB = GSS_WARP_BITONIC && !KV && BitwiseOrder<Cmp>::value && !BITONIC;
 

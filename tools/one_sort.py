@@ -20,13 +20,17 @@ ap.add_argument("--k", type=int, default=0)                 # 0: the library def
 ap.add_argument("--tile", type=int, default=0)                # 0: the library default
 ap.add_argument("--M", type=int, default=0)
 ap.add_argument("--fill_div", type=int, default=0)
+ap.add_argument("--flags", type=int, default=0)
+ap.add_argument("--cls_arrays", type=int, default=0)
+ap.add_argument("--a", type=int, default=0)
 args = ap.parse_args()
 n, bits, pairs, dist, _ = bench.WORKLOADS[args.workload]
 x = inputs.keys(dist, n, bits, seed=1)
 k = torch.from_numpy(x).cuda()
 v = torch.from_numpy(inputs.values(n, bits)).cuda() if pairs else None
 M = args.M or (8192 if (pairs and bits == 64) else (32768 if (bits == 32 and not pairs) else 16384))
-s = gss.Sorter(f"u{bits}", n, pairs, k=args.k, tile=args.tile, M=M, fill_div=args.fill_div or None)
+s = gss.Sorter(f"u{bits}", n, pairs, k=args.k, tile=args.tile, M=M, fill_div=args.fill_div or None, flags=args.flags,
+               cls_arrays=args.cls_arrays or None, a=args.a or None)
 ko = torch.empty_like(k)
 vo = torch.empty_like(v) if pairs else None
 for i in range(args.warmup + args.steps):
