@@ -16,3 +16,5 @@ run scatter_regs k_scatter 1 --flags 32
 run scatter_direct k_scatter 1 --flags 8
 run small_oem k_small_block 4
 run small_bitonic k_small_block 4 --flags 128
+python tools/summarize_ablations.py $TAG > gpurun_out/abl_${TAG}_summarize.log 2>&1
+rm -f gpurun_out/abl_${TAG}_*.ncu-rep     # gpurun_out/ comes back only under 64 MiB
