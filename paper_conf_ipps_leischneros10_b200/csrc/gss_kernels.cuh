@@ -29,6 +29,9 @@ constexpr int kClsThreads = 256;
 #ifndef GSS_SCATTER_EARLY
 #define GSS_SCATTER_EARLY 0
 #endif
+#ifndef GSS_SCATTER_SPREAD
+#define GSS_SCATTER_SPREAD 1     // per-id work of the scatter spread over every warp (0: the first kmax threads)
+#endif
 #ifndef GSS_SCATTER_PAIRFOLD
 #define GSS_SCATTER_PAIRFOLD 0   // 1: two threads per id in the fold (u64 3.18 vs 3.11 ms, pairs 3.30 vs 2.99: slower)
 #endif
@@ -814,8 +817,12 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
     } else
 #endif
     {
-      const uint32_t per = (cur_K + kScatterThreads - 1) / kScatterThreads;
-      const uint32_t i0 = threadIdx.x * per;
+      // id owners spread over every warp (thread i * threads/kmax owns id i), in thread order for the scan
+      const bool spread = GSS_SCATTER_SPREAD && kmax <= (uint32_t)kScatterThreads;
+      const uint32_t sstride = spread ? (uint32_t)kScatterThreads / kmax : 1u;
+      const uint32_t per = spread ? ((threadIdx.x % sstride) == 0 ? 1u : 0u)
+                                  : (cur_K + kScatterThreads - 1) / kScatterThreads;
+      const uint32_t i0 = spread ? threadIdx.x / sstride : threadIdx.x * per;
       uint32_t tsum = 0;
       for (uint32_t j = 0; j < per; j++) {
         const uint32_t id = i0 + j;
@@ -1025,8 +1032,15 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     idb = B.id_base + tl * c.T;
   };
   // ids owned by this thread in the scan and the write phase, fixed for the
-  // kernel (gbase, rstart, rlen of an id are only touched by its owner)
-  const uint32_t per = (kmax + kScatterThreads - 1) / kScatterThreads, i0 = threadIdx.x * per;
+  // kernel (gbase, rstart, rlen of an id are only touched by its owner).
+  // With kmax <= threads, id i belongs to thread i * (threads / kmax): the
+  // owners (and their serialised bulk copies) are spread over every warp,
+  // in thread order, as the scan requires.
+  const bool spread = GSS_SCATTER_SPREAD && kmax <= (uint32_t)kScatterThreads;
+  const uint32_t sstride = spread ? (uint32_t)kScatterThreads / kmax : 1u;
+  const uint32_t per = spread ? ((threadIdx.x % sstride) == 0 ? 1u : 0u)
+                              : (kmax + kScatterThreads - 1) / kScatterThreads;
+  const uint32_t i0 = spread ? threadIdx.x / sstride : threadIdx.x * per;
   auto load_gbase = [&](uint32_t tt) {                            // owner threads only: no barrier needed
     const Bucket B = c.bk[slot][c.tile_bucket[slot][tt]];
     const uint32_t tl = tt - B.tile_start;
