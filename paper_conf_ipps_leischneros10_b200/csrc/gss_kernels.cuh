@@ -30,7 +30,7 @@ constexpr int kClsThreads = 256;
 #define GSS_SCATTER_EARLY 0
 #endif
 #ifndef GSS_SCATTER_SPREAD
-#define GSS_SCATTER_SPREAD 1     // per-id work of the scatter spread over every warp (0: the first kmax threads)
+#define GSS_SCATTER_SPREAD 0     // 1: per-id work spread over every warp -- measured slower (2^28 u64 scatter 3.16 vs 2.94 ms)
 #endif
 #ifndef GSS_SCATTER_PAIRFOLD
 #define GSS_SCATTER_PAIRFOLD 0   // 1: two threads per id in the fold (u64 3.18 vs 3.11 ms, pairs 3.30 vs 2.99: slower)
@@ -586,6 +586,26 @@ __device__ __forceinline__ uint32_t atom_add_shared_if(uint32_t pred, uint32_t s
   return old;
 }
 
+// Rank of a key within (warp, id) from the warp's counters; returns (rank << 16) | id, or the empty
+// marker.  One shared atomic per key -- except when the whole warp holds one id (sorted input,
+// long equal runs, few distinct keys), where 32 atomics on one address would serialise: then lane
+// 0 adds 32 and the lanes take ranks in lane order (deterministic either way).
+__device__ __forceinline__ uint32_t rank_in_warp(uint32_t iid, uint32_t wc_s, int lane) {
+  const uint32_t id = iid & 0xffffu;
+#ifndef GSS_WARP_UNIFORM_RANK
+#define GSS_WARP_UNIFORM_RANK 1
+#endif
+  const uint32_t first = __shfl_sync(kFull, iid, 0);
+  if (GSS_WARP_UNIFORM_RANK && __all_sync(kFull, iid == first && iid != 0xffffffffu)) {
+    uint32_t base = 0;
+    if (lane == 0) base = atom_add_shared_if(1u, wc_s + 4 * id, 32u);
+    base = __shfl_sync(kFull, base, 0);
+    return ((base + (uint32_t)lane) << 16) | id;
+  }
+  const uint32_t r = atom_add_shared_if(iid != 0xffffffffu ? 1u : 0u, wc_s + 4 * id, 1u);
+  return iid == 0xffffffffu ? iid : (r << 16) | id;
+}
+
 // Phase 4 kernel.  Persistent: the CTA walks its tiles (blockIdx.x, +gridDim.x,
 // ...) chunk by chunk; the keys, values and ids of the next chunk are loaded
 // into registers before the current chunk's runs are written out, so the
@@ -781,10 +801,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB) k_scatter(C
       // unique within (warp, id) in any order, so the level is a partition
       // whose within-bucket order is the hardware's atomic order.
 #pragma unroll
-      for (int it = 0; it < kScatterIter; it++) {
-        const uint32_t r = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (iid[it] & 0xffffu), 1u);
-        iid[it] = iid[it] == 0xffffffffu ? iid[it] : (r << 16) | iid[it];
-      }
+      for (int it = 0; it < kScatterIter; it++) iid[it] = rank_in_warp(iid[it], wc_s, lane);
     }
     __syncthreads();
     GSS_PH(0);
@@ -1091,10 +1108,7 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
     }
     // ranks within (warp, id): one shared atomic per key on the warp's own counters
 #pragma unroll
-    for (int it = 0; it < kScatterIter; it++) {
-      const uint32_t r = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (iid[it] & 0xffffu), 1u);
-      iid[it] = iid[it] == 0xffffffffu ? iid[it] : (r << 16) | iid[it];
-    }
+    for (int it = 0; it < kScatterIter; it++) iid[it] = rank_in_warp(iid[it], wc_s, lane);
     // the staging buffer written below was last read by the copies issued NBUF chunks ago
     bulk_wait_read<NBUF - 1>();
     __syncthreads();                                                // B1: counters complete
