@@ -14,7 +14,7 @@ ap.add_argument("--dist", default=None, help="override the workload's input dist
 ap.add_argument("cfgs", nargs="*")
 a = ap.parse_args()
 n, bits, pairs, dist, _ = bench.WORKLOADS[a.workload]
-dist = a.dist or dist
+dist = a.dist or os.environ.get("GSS_DIST") or dist
 x = inputs.keys(dist, n, bits, seed=1)
 k = torch.from_numpy(x).cuda()
 v = torch.from_numpy(inputs.values(n, bits)).cuda() if pairs else None
