@@ -2235,17 +2235,41 @@ __global__ void __launch_bounds__(kSplitMaxThreads, 2)
 
 // Final equality buckets larger than the in-SM capacity that did not end in
 // keys_out: moved tile by tile.
+// dst[0..m) = src[0..m) by one CTA: 16-byte vectors (source and destination share their alignment:
+// the same index of two 256-byte aligned buffers) with four in flight per thread, scalar ends.
+template <class T>
+__device__ __forceinline__ void cta_copy(T* __restrict__ dst, const T* __restrict__ src, uint32_t m) {
+  constexpr uint32_t A = 16 / sizeof(T);
+  const uint32_t mis = (uint32_t)((reinterpret_cast<uintptr_t>(src) & 15u) / sizeof(T));
+  const uint32_t head = min(m, (A - mis) & (A - 1));
+  const uint32_t nv = (m - head) / A;
+  for (uint32_t q = threadIdx.x; q < head; q += blockDim.x) dst[q] = src[q];
+  const uint4* vs = reinterpret_cast<const uint4*>(src + head);
+  uint4* vd = reinterpret_cast<uint4*>(dst + head);
+  constexpr int U = 4;
+  for (uint32_t q0 = threadIdx.x; q0 < nv; q0 += U * blockDim.x) {
+    uint4 t[U];
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const uint32_t q = q0 + u * blockDim.x;
+      if (q < nv) t[u] = vs[q];
+    }
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const uint32_t q = q0 + u * blockDim.x;
+      if (q < nv) vd[q] = t[u];
+    }
+  }
+  for (uint32_t q = head + nv * A + threadIdx.x; q < m; q += blockDim.x) dst[q] = src[q];
+}
+
 template <class Key, class Val, class IdT>
 __global__ void k_copy(Ctx<Key, Val, IdT> c) {
   const uint32_t ni = min(c.cnt->copy_count, c.cap_copy);
   for (uint32_t i = blockIdx.x; i < ni; i += gridDim.x) {
     const Item I = c.copy[i];
-    const Key* ks = c.keys(I.buf);
-    for (uint32_t q = threadIdx.x; q < I.m; q += blockDim.x) c.kout[I.lo + q] = ks[I.lo + q];
-    if constexpr (kHasVal<Val>) {
-      const Val* vs = c.vals(I.buf);
-      for (uint32_t q = threadIdx.x; q < I.m; q += blockDim.x) c.vout[I.lo + q] = vs[I.lo + q];
-    }
+    cta_copy(c.kout + I.lo, c.keys(I.buf) + I.lo, I.m);
+    if constexpr (kHasVal<Val>) cta_copy(c.vout + I.lo, c.vals(I.buf) + I.lo, I.m);
   }
 }
 
