@@ -705,3 +705,76 @@ def test_error_out_flags(gss):
         s(kin, kout)
         assert int(err.item()) == 0
     np.testing.assert_array_equal(to_host(kout), np.sort(x))
+
+
+# ---------------------------------------------------------------------------
+# The fused global scatter with several destination segments (the P > 1 data path of
+# GSS_FLAG_DIST_FUSED, which a world-size-1 run cannot reach: there the only segment is the
+# rank's own window).  gssi_dist_level (internal export): phase 1 classifies and counts, phase 2
+# scatters the equality-mode partition straight into P separate buffers through a RemoteSeg table
+# whose cuts fall anywhere (inside buckets too); every bucket must arrive whole, as a multiset.
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("P", [2, 3, 8])
+def test_fused_scatter_segments(gss, width, pairs, P):
+    import ctypes
+    lib = gss._lib()
+    fn = getattr(lib, f"gssi_dist_level_u{width}")
+    vp, sz, u32 = ctypes.c_void_p, ctypes.c_size_t, ctypes.c_uint32
+    fn.restype = ctypes.c_int
+    fn.argtypes = [vp, vp, vp, vp, sz, vp, u32, vp, vp, u32, u32, vp, ctypes.POINTER(sz), vp]
+    n = 3 * 65536 + 4321
+    x = inputs.keys("and3", n, width, seed=P)
+    v = inputs.values(n, width)
+    rng = np.random.default_rng(P)
+    spl = np.sort(x[rng.integers(0, n, size=P - 1)])
+    nspl = P - 1
+    b = np.searchsorted(spl, x, side="left")
+    ids = 2 * b + ((b < nspl) & (x == spl[np.minimum(b, nspl - 1)]))
+    order = np.argsort(ids, kind="stable")
+    want_k, want_v, want_ids = x[order], v[order], ids[order]
+    # P segments with arbitrary cuts of the partition index space, each into its own buffer at an offset
+    cuts = np.sort(np.concatenate([[0, n], rng.integers(0, n, size=P - 1)]))
+    dt = DT[width]
+    kin, vin = to_dev(x), to_dev(v)
+    kbuf, vbuf = torch.empty_like(kin), torch.empty_like(vin)           # stand-in local output (unused)
+    dspl = to_dev(spl)
+    cnt = torch.zeros(2 * nspl + 1, dtype=torch.uint64, device="cuda")
+    outs, offs = [], []
+    seg = np.zeros((P, 4), dtype=np.uint64)                             # (lo|hi, pad, kdst, vdst) as u64 words
+    w = width // 8
+    for q in range(P):
+        lo, hi = int(cuts[q]), int(cuts[q + 1])
+        off = 7 * q + 3                                                  # arbitrary alignment of the destination
+        kd = torch.zeros(hi - lo + off + 8, dtype=dt, device="cuda")
+        vd = torch.zeros(hi - lo + off + 8, dtype=dt, device="cuda")
+        outs.append((kd, vd)); offs.append(off)
+        seg[q, 0] = np.uint64(lo | (hi << 32))
+        seg[q, 2] = np.uint64((kd.data_ptr() + (off - lo) * w) % (1 << 64))
+        seg[q, 3] = np.uint64((vd.data_ptr() + (off - lo) * w) % (1 << 64)) if pairs else 0
+    dseg = torch.from_numpy(seg.view(np.int64)).cuda()
+    head = (ctypes.c_void_p(kin.data_ptr()), ctypes.c_void_p(vin.data_ptr()) if pairs else None,
+            ctypes.c_void_p(kbuf.data_ptr()), ctypes.c_void_p(vbuf.data_ptr()) if pairs else None, n,
+            ctypes.c_void_p(dspl.data_ptr()), nspl, ctypes.c_void_p(cnt.data_ptr()))
+    tb = sz(0)
+    assert fn(*head, None, 0, 1, None, ctypes.byref(tb), None) == 0
+    temp = torch.empty(max(tb.value, 1), dtype=torch.uint8, device="cuda")
+    s = torch.cuda.current_stream().cuda_stream
+    assert fn(*head, None, 0, 1, ctypes.c_void_p(temp.data_ptr()), ctypes.byref(tb), s) == 0
+    assert fn(*head, ctypes.c_void_p(dseg.data_ptr()), P, 2, ctypes.c_void_p(temp.data_ptr()), ctypes.byref(tb), s) == 0
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(to_host(cnt), np.bincount(ids, minlength=2 * nspl + 1))
+    got_k = np.concatenate([to_host(outs[q][0])[offs[q]:offs[q] + int(cuts[q + 1] - cuts[q])] for q in range(P)])
+    got_v = np.concatenate([to_host(outs[q][1])[offs[q]:offs[q] + int(cuts[q + 1] - cuts[q])] for q in range(P)])
+    # bucket by bucket, the same (key, value) multiset as the stable partition
+    bounds = np.concatenate([[0], np.cumsum(np.bincount(ids, minlength=2 * nspl + 1))])
+    for i in range(2 * nspl + 1):
+        a, e = int(bounds[i]), int(bounds[i + 1])
+        if pairs:
+            np.testing.assert_array_equal(np.sort(got_v[a:e]), np.sort(want_v[a:e]))
+            np.testing.assert_array_equal(x[got_v[a:e].astype(np.int64)], got_k[a:e])
+        else:
+            np.testing.assert_array_equal(np.sort(got_k[a:e]), np.sort(want_k[a:e]))
+    for q in range(P):                                                   # nothing written outside the segments
+        kd = to_host(outs[q][0])
+        assert not kd[:offs[q]].any() and not kd[offs[q] + int(cuts[q + 1] - cuts[q]):].any()
