@@ -778,3 +778,46 @@ def test_fused_scatter_segments(gss, width, pairs, P):
     for q in range(P):                                                   # nothing written outside the segments
         kd = to_host(outs[q][0])
         assert not kd[:offs[q]].any() and not kd[offs[q] + int(cuts[q + 1] - cuts[q]):].any()
+
+
+@pytest.mark.parametrize("width,pairs", KINDS)
+@pytest.mark.parametrize("P,dist_name", [(2, "uniform"), (4, "dd"), (8, "staggered"), (8, "equal")])
+def test_distributed_steps_virtual_ranks(gss, oracle_mod, width, pairs, P, dist_name):
+    """The distributed sort's device steps for P virtual ranks on one GPU, composed exactly as
+    gss_dist_sort does (only the collectives are replaced by device copies): hashed samples of every
+    shard (gss_sample, level tag 255, lo = shard start), the sorted gathered sample (gss_sort), the
+    splitters S[(i+1)VS/P - 1], the equality-mode partition of every shard (gss_partition_by_eq), the
+    exchange plan (gss_dist_plan), the exchange, the local sorts.  The concatenation over ranks equals
+    the oracle's sort of the global input; duplicate-heavy inputs stay balanced."""
+    from paper_conf_ipps_leischneros10_b200.dist import plan
+    n_local, S = (1 << 18) + 77, 16384
+    x = inputs.keys(dist_name, n_local * P, width, seed=5)
+    v = inputs.values(n_local * P, width)
+    shards = [(to_dev(x[r * n_local:(r + 1) * n_local]), to_dev(v[r * n_local:(r + 1) * n_local])) for r in range(P)]
+    smp = torch.cat([gss.sample(k, S, lo_global=r * n_local, level_tag=255, seed=5489) for r, (k, _) in enumerate(shards)])
+    ssorted, _ = gss.sort(smp)
+    VS = P * S
+    spl = ssorted[torch.tensor([((i + 1) * VS) // P - 1 for i in range(P - 1)], dtype=torch.long, device="cuda")]
+    parts = [gss.partition_by(k, vv if pairs else None, spl, eq=True) for k, vv in shards]
+    counts = np.stack([to_host(c).astype(np.uint64) for _, _, c in parts])
+    plans = [plan(P, r, counts) for r in range(P)]
+    results = []
+    for q in range(P):                                          # rank q receives, source-major, then sorts
+        rk, rv = [], []
+        for r in range(P):
+            so, sc = int(plans[r][1][q]), int(plans[r][2][q])
+            rk.append(parts[r][0][so:so + sc])
+            if pairs:
+                rv.append(parts[r][1][so:so + sc])
+            assert sc == int(plans[q][3][r])                   # what r sends to q is what q expects from r
+        kq = torch.cat(rk)
+        vq = torch.cat(rv) if pairs else None
+        ko, vo = gss.sort(kq, vq)
+        results.append((to_host(ko), to_host(vo) if pairs else None))
+    ok, _, _ = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=4096))
+    got = np.concatenate([r[0] for r in results])
+    np.testing.assert_array_equal(got, ok)
+    if pairs:
+        check_pairs(x, np.concatenate([r[1] for r in results]), ok)
+    for r in results:                                           # balanced to within a few percent
+        assert abs(len(r[0]) - n_local) <= 0.1 * n_local, [len(t[0]) for t in results]
