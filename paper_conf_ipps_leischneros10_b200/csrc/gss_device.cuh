@@ -458,7 +458,30 @@ struct CtaSort {
   static constexpr bool kFastMerge = !KV && std::is_same<Cmp, Less>::value && std::is_unsigned<Key>::value &&
                                      (sizeof(Key) == 4 || sizeof(Key) == 8);
   __device__ static __forceinline__ void fast_step(Key& out, Key& ka, Key& kb, int& xa, int& xb, uint32_t sb) {
-    if constexpr (sizeof(Key) == 8) {
+#ifndef GSS_MERGE_ONELOAD
+#define GSS_MERGE_ONELOAD 0
+#endif
+    if constexpr (GSS_MERGE_ONELOAD && sizeof(Key) == 8) {
+      // one shared load with every lane active (the consumed head's successor), then selects: one
+      // instruction of up to 32 random 8-byte addresses instead of two complementary predicated ones
+      unsigned long long o, a = ka, b = kb;
+      asm volatile(
+          "{\n\t.reg .pred p;\n\t.reg .u32 x, t;\n\t.reg .u64 y;\n\t"
+          "setp.ge.u64 p, %1, %2;\n\t"
+          "selp.b64 %0, %2, %1, p;\n\t"
+          "@!p add.s32 %3, %3, 1;\n\t"
+          "@p add.s32 %4, %4, -1;\n\t"
+          "selp.b32 x, %4, %3, p;\n\t"
+          "shr.s32 t, x, 4;\n\t"
+          "add.s32 t, t, x;\n\t"
+          "mad.lo.u32 t, t, 8, %5;\n\t"
+          "ld.volatile.shared.u64 y, [t];\n\t"
+          "selp.b64 %1, %1, y, p;\n\t"
+          "selp.b64 %2, y, %2, p;\n\t}"
+          : "=l"(o), "+l"(a), "+l"(b), "+r"(xa), "+r"(xb)
+          : "r"(sb));
+      out = (Key)o; ka = (Key)a; kb = (Key)b;
+    } else if constexpr (sizeof(Key) == 8) {
       unsigned long long o, a = ka, b = kb;
       asm volatile(
           "{\n\t.reg .pred p;\n\t.reg .u32 x, t;\n\t"
