@@ -797,7 +797,9 @@ def test_distributed_steps_virtual_ranks(gss, oracle_mod, width, pairs, P, dist_
     smp = torch.cat([gss.sample(k, S, lo_global=r * n_local, level_tag=255, seed=5489) for r, (k, _) in enumerate(shards)])
     ssorted, _ = gss.sort(smp)
     VS = P * S
-    spl = ssorted[torch.tensor([((i + 1) * VS) // P - 1 for i in range(P - 1)], dtype=torch.long, device="cuda")]
+    sdt = torch.int32 if width == 32 else torch.int64                    # (no unsigned gather on CUDA in torch)
+    pos = torch.tensor([((i + 1) * VS) // P - 1 for i in range(P - 1)], dtype=torch.long, device="cuda")
+    spl = ssorted.view(sdt)[pos].view(ssorted.dtype)
     parts = [gss.partition_by(k, vv if pairs else None, spl, eq=True) for k, vv in shards]
     counts = np.stack([to_host(c).astype(np.uint64) for _, _, c in parts])
     plans = [plan(P, r, counts) for r in range(P)]
