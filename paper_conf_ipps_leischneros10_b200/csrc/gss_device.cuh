@@ -461,6 +461,9 @@ struct CtaSort {
 #ifndef GSS_MERGE_ONELOAD
 #define GSS_MERGE_ONELOAD 1   // 0: two complementary predicated loads (2^28 u64 in-SM sort 4.89 vs 4.79 ms)
 #endif
+#ifndef GSS_MERGE_ONELOAD32
+#define GSS_MERGE_ONELOAD32 0 // 4-byte keys: 1 measured slower (2^27 u32 in-SM sort 1.63 vs 1.61 ms)
+#endif
     if constexpr (GSS_MERGE_ONELOAD && sizeof(Key) == 8) {
       // one shared load with every lane active (the consumed head's successor), then selects: one
       // instruction of up to 32 random 8-byte addresses instead of two complementary predicated ones
@@ -481,7 +484,7 @@ struct CtaSort {
           : "=l"(o), "+l"(a), "+l"(b), "+r"(xa), "+r"(xb)
           : "r"(sb));
       out = (Key)o; ka = (Key)a; kb = (Key)b;
-    } else if constexpr (GSS_MERGE_ONELOAD && sizeof(Key) == 4) {
+    } else if constexpr (GSS_MERGE_ONELOAD32 && sizeof(Key) == 4) {
       uint32_t o, a = ka, b = kb;
       asm volatile(
           "{\n\t.reg .pred p;\n\t.reg .u32 x, t, y;\n\t"
