@@ -148,6 +148,13 @@ typedef struct gss_params {
                                       shared memory (the on-chip answer to the
                                       paper's quicksort tier below M = 2^17); the
                                       default M becomes the cluster capacity (8x the CTA's)  */
+#define GSS_FLAG_TREE_CLASSIFY 512u /* unsigned keys under operator<: Phase 2 classifies every key
+                                      by the paper's branch-free descent of the splitter tree
+                                      (Algorithm 2) instead of the default
+                                      radix-indexed lookup (a table of 4096 key-value bins per
+                                      bucket, one shared load per key, the descent only inside
+                                      bins that hold a splitter); both give identical ids
+                                      (ablation)                                             */
 #define GSS_FLAG_SPLIT_SORT 2u     /* finish buckets of two or more warps with one more
                                       sample-sort split inside the SM + warp merge sorts of
                                       packed segments; ablation: on B200 its

@@ -25,6 +25,7 @@ __all__ = ["sort", "sort_host", "Sorter", "HostSorter", "HostPipeline", "partiti
 KERNEL_KINDS = ["init", "sample", "classify", "scan", "scatter", "plan", "small_sort", "copy", "overflow", "h2d",
                 "d2h", "other"]
 FLAG_RECOMPUTE_IDS = 1
+FLAG_TREE_CLASSIFY = 512
 
 _u32, _u64, _vp, _sz = ctypes.c_uint32, ctypes.c_uint64, ctypes.c_void_p, ctypes.c_size_t
 

@@ -139,6 +139,7 @@ struct Ctx {
   uint32_t nremote;
   uint32_t n, M, T, k, a, k_policy, fill_div, sample_cap, L, mode, dst0, src0, stable;
   uint32_t recompute;                // GSS_FLAG_RECOMPUTE_IDS: no stored ids, Phase 4 re-descends
+  uint32_t lut;                      // radix-indexed splitter lookup in Phase 2 (off: GSS_FLAG_TREE_CLASSIFY)
   uint32_t cap_buckets, cap_tiles, cap_hist, cap_spl, cap_copy, cap_ovf, cap_fb, cap_clus;
   uint32_t cap_small[kNumClasses];
   uint32_t class_cap[kNumClasses];

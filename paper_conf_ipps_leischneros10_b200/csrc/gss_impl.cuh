@@ -299,6 +299,7 @@ struct Engine {
     c.stable = ((cfg.flags & GSS_FLAG_STABLE) || mode != MODE_SORT) ? 1u : 0u;   // partitions stay stable (R7 probe)
     c.recompute = (!c.stable && (cfg.flags & GSS_FLAG_RECOMPUTE_IDS) && !(cfg.flags & GSS_FLAG_DIRECT_SCATTER) &&
                    !(cfg.flags & kFlagScatterCtaCounters)) ? 1u : 0u;
+    c.lut = (cfg.flags & GSS_FLAG_TREE_CLASSIFY) ? 0u : 1u;
     c.cap_buckets = lay.cap_buckets; c.cap_tiles = lay.cap_tiles; c.cap_hist = lay.cap_hist;
     c.cap_spl = lay.cap_spl; c.cap_copy = lay.cap_copy; c.cap_ovf = lay.cap_ovf;
     c.cap_fb = lay.cap_fb;
@@ -355,6 +356,9 @@ struct Engine {
     auto ks = k_sample<Key, Val, IdT, Cmp>;
     const size_t sm_sample = CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
     auto kc = mode == MODE_PARTITION_BY ? k_classify<Key, Val, IdT, Cmp, true> : k_classify<Key, Val, IdT, Cmp, false>;
+    if constexpr (lut_ok<Key, Cmp>()) {
+      if (mode != MODE_PARTITION_BY && c.lut) kc = k_classify<Key, Val, IdT, Cmp, false, true>;   // radix-indexed lookup
+    }
     const size_t sm_cls = cls_smem_bytes<Key>(kmax);
     auto ksc = c.stable ? k_scatter<Key, Val, IdT, Cmp, true>
                         : (c.recompute ? k_scatter<Key, Val, IdT, Cmp, false, true> : k_scatter<Key, Val, IdT, Cmp, false>);

@@ -247,7 +247,7 @@ constexpr uint32_t rep_copies() { return 128u / sizeof(Key); }
 template <class Key>
 constexpr size_t cls_smem_bytes(uint32_t kmax) {
   return (size_t)kmax * sizeof(Key) * 2 + (size_t)kRepNodes * 128 + (size_t)(kClsThreads / 32) * kmax * 4 +
-         (size_t)(kClsThreads / 32) * (32 * GSS_CLS_U) * 2;
+         (size_t)(kClsThreads / 32) * (32 * GSS_CLS_U) * 2 + (size_t)(1u << 12) * 4 + 64 * 4;   // + lookup table, scan scratch
 }
 
 // One level of Algorithm 2 (j := 2j + (e > bt[j])) on a node address
@@ -340,16 +340,149 @@ __device__ __forceinline__ void descend_group(const Key (&e)[U], uint32_t (&id)[
   }
 }
 
+// ---------------------------------------------------------------------------
+// Radix-indexed splitter lookup: an exact replacement of the descent for
+// unsigned keys under operator< (the same id b = #{splitters s < e} that
+// Algorithm 2 computes).  The bucket's splitter range
+// [s_0, s_{ks-2}] is cut into kLutN bins of 2^shift key values each (keys
+// below s_0 fall into bin 0, keys above the range into the last, open bin);
+// lut[i] = lo | hi << 16 with lo = #{s < start of bin i} and hi = #{s < end
+// of bin i}.  A key of bin i has lo <= b <= hi: when lo == hi -- every bin
+// without a splitter, i.e. all but at most ks-1 of the kLutN -- the single
+// shared load is the whole classification; otherwise spl[lo] decides between
+// lo and lo+1, and a bin holding two or more splitters (rare unless the keys
+// cluster in value) finishes with a binary search over spl[lo+1 .. hi).  On
+// B200 the 8-level descent is issue-bound (~65 instructions per u64 key); the
+// lookup needs about a third of that.  GSS_FLAG_TREE_CLASSIFY keeps the
+// paper's descent for every key (ablation).
+// ---------------------------------------------------------------------------
+constexpr uint32_t kLutBits = 12, kLutN = 1u << kLutBits;
+template <class Key, class Cmp>
+constexpr bool lut_ok() { return std::is_same<Cmp, Less>::value && std::is_unsigned<Key>::value; }
+
+template <class Key>
+__device__ __forceinline__ uint32_t lut_bin(Key e, Key base, uint32_t shift) {
+  const Key q = (Key)(e - base) >> shift;
+  const uint32_t i = q > (Key)(kLutN - 1) ? kLutN - 1 : (uint32_t)q;
+  return e < base ? 0u : i;
+}
+
+// Builds lut[0..kLutN) from the nspl sorted splitters in shared memory; every
+// thread of the kClsThreads-thread CTA calls it (begins and ends with a barrier).
+// Returns whether the table pays for this bucket: false when more than 1/8 of
+// the splitters share a bin with another one (keys clustered in value, e.g.
+// AND-ed random words, whose splitters crowd the low bins) -- those buckets
+// keep the descent.
+template <class Key>
+__device__ __forceinline__ bool lut_build(uint32_t* lut, const Key* spl, uint32_t nspl, Key& base, uint32_t& shift,
+                                          uint32_t* s_warp) {
+  constexpr uint32_t PER = kLutN / kClsThreads;
+  static_assert(PER * kClsThreads == kLutN, "bins per thread");
+  __syncthreads();                                             // spl[] is loaded
+  base = nspl ? spl[0] : Key(0);
+  const Key span = nspl ? (Key)(spl[nspl - 1] - base) : Key(0);
+  uint32_t bl = 0;
+  if constexpr (sizeof(Key) == 8) bl = span ? 64u - (uint32_t)__clzll((long long)span) : 0u;
+  else bl = span ? 32u - (uint32_t)__clz((int)span) : 0u;
+  shift = bl > kLutBits ? bl - kLutBits : 0u;
+#pragma unroll
+  for (uint32_t j = 0; j < PER; j++) lut[threadIdx.x + j * kClsThreads] = 0;
+  if (threadIdx.x == 0) s_warp[63] = 0;
+  __syncthreads();
+  for (uint32_t j = threadIdx.x; j < nspl; j += kClsThreads) atomicAdd(lut + lut_bin(spl[j], base, shift), 1u);
+  __syncthreads();
+  uint32_t cnt[PER], tot = 0, crowd = 0;
+#pragma unroll
+  for (uint32_t j = 0; j < PER; j++) {
+    cnt[j] = lut[threadIdx.x * PER + j];
+    tot += cnt[j];
+    crowd += cnt[j] >= 2 ? cnt[j] : 0u;
+  }
+  if (crowd) atomicAdd(s_warp + 63, crowd);
+  uint32_t lo = block_exclusive_scan<kClsThreads>(tot, s_warp, nullptr);   // ends with a barrier
+#pragma unroll
+  for (uint32_t j = 0; j < PER; j++) {
+    lut[threadIdx.x * PER + j] = lo | ((lo + cnt[j]) << 16);
+    lo += cnt[j];
+  }
+  const bool good = s_warp[63] * 8 <= nspl;
+  __syncthreads();
+  return good;
+}
+
+// Bucket ids of U keys per lane by the lookup, then the id rule of the tile's
+// mode (0: range buckets, 1: equality mode R4), as in descend_group.
+template <int MODE, int U, class Key>
+__device__ __forceinline__ void lut_group(const Key (&e)[U], uint32_t (&id)[U], uint32_t lut_s, const Key* spl,
+                                          Key base, uint32_t shift, uint32_t ks) {
+  uint32_t b[U], slow = 0;
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    uint32_t ent;
+    asm volatile("ld.shared.u32 %0, [%1];" : "=r"(ent) : "r"(lut_s + 4u * lut_bin(e[u], base, shift)));
+    const uint32_t lo = ent & 0xffffu, hi = ent >> 16;
+    b[u] = lo;
+    if (hi > lo) {
+      const bool gt = spl[lo] < e[u];
+      b[u] = lo + (gt ? 1u : 0u);
+      if (gt && hi > lo + 1) slow |= 1u << u;
+    }
+  }
+  if (__any_sync(kFull, slow)) {
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      if (slow & (1u << u)) {
+        // first index of spl[b .. hi) not below e (the bin's remaining splitters)
+        uint32_t l = b[u], h;
+        {
+          uint32_t ent;
+          asm volatile("ld.shared.u32 %0, [%1];" : "=r"(ent) : "r"(lut_s + 4u * lut_bin(e[u], base, shift)));
+          h = ent >> 16;
+        }
+        while (l < h) {
+          const uint32_t m = (l + h) >> 1;
+          if (spl[m] < e[u]) l = m + 1; else h = m;
+        }
+        b[u] = l;
+      }
+    }
+  }
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    if constexpr (MODE == 1) {
+      const uint32_t bb = min(b[u], ks - 2);
+      id[u] = 2 * b[u] + ((b[u] + 1 < ks && !(e[u] < spl[bb])) ? 1u : 0u);
+    } else {
+      id[u] = b[u];
+    }
+  }
+}
+
+// Where a tile's ids come from: the descent (tree_s, rep_b, logk) or the lookup (lut_s, base, shift).
+template <class Key>
+struct ClsSrc {
+  uint32_t tree_s, rep_b, logk, lut_s, shift;
+  Key base;
+  bool use_lut;                      // this bucket classifies by the lookup (else the descent)
+};
+
 // Warp-contiguous groups: warp w of the CTA handles keys [g + 256 w, g + 256 w
 // + 256) of each 2048-key group g, lane l the keys 32u + l (coalesced loads);
 // the warp stages its 256 ids in shared memory and writes them as one 8-byte
 // store per lane.  Full groups run without bounds tests; the next group's
 // keys are loaded before this group descends.
-template <int MODE, bool STORE, class Key, class IdT, class Cmp>
+template <int MODE, bool STORE, bool LUT, class Key, class IdT, class Cmp>
 __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* __restrict__ tids, uint32_t beg,
-                                              uint32_t len, uint32_t tree_s, uint32_t rep_b, const Key* spl,
-                                              uint32_t logk, uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid,
-                                              Cmp less) {
+                                              uint32_t len, const ClsSrc<Key>& cs, const Key* spl,
+                                              uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid, Cmp less) {
+  auto ids_of = [&](const Key (&e)[GSS_CLS_U], uint32_t (&id)[GSS_CLS_U]) {
+    if constexpr (LUT) {
+      if (cs.use_lut) lut_group<MODE>(e, id, cs.lut_s, spl, cs.base, cs.shift, ks);
+      else descend_group<MODE>(e, id, cs.tree_s, cs.rep_b, spl, cs.logk, ks, K, less);
+    } else {
+      descend_group<MODE>(e, id, cs.tree_s, cs.rep_b, spl, cs.logk, ks, K, less);
+    }
+  };
   constexpr int U = GSS_CLS_U;                                 // keys per lane per group
   constexpr uint32_t G = U * kClsThreads;                      // keys per group
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
@@ -370,7 +503,7 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
       for (int u = 0; u < U; u++) nx[u] = sp[(g + 1) * G + u * 32];
     }
     uint32_t id[U];
-    descend_group<MODE>(e, id, tree_s, rep_b, spl, logk, ks, K, less);
+    ids_of(e, id);
 #pragma unroll
     for (int u = 0; u < U; u++) {
       red_shared_add(wc_s + 4 * id[u], 1u);
@@ -404,7 +537,7 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
       else e[u] = src[beg];
     }
     uint32_t id[U];
-    descend_group<MODE>(e, id, tree_s, rep_b, spl, logk, ks, K, less);
+    ids_of(e, id);
 #pragma unroll
     for (int u = 0; u < U; u++) {
       const uint32_t i = tb + off + u * 32;
@@ -421,7 +554,7 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
 // memory.
 // PART: the partition_by modes (2, 3) only; else the sort modes (0, 1): each
 // instantiation holds only the descents it runs (their registers add up).
-template <class Key, class Val, class IdT, class Cmp, bool PART = false>
+template <class Key, class Val, class IdT, class Cmp, bool PART = false, bool LUT = false>
 #ifndef GSS_CLS_MINB
 #define GSS_CLS_MINB 2
 #endif
@@ -433,7 +566,10 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
   Key* rep = spl + kmax;                                       // kRepNodes x REP keys
   uint32_t* wcnt = reinterpret_cast<uint32_t*>(rep + kRepNodes * REP);
   constexpr int NW = kClsThreads / 32;
-  IdT* wid = reinterpret_cast<IdT*>(wcnt + NW * kmax) + (threadIdx.x >> 5) * (32 * GSS_CLS_U);   // per-warp id staging
+  IdT* wid0 = reinterpret_cast<IdT*>(wcnt + NW * kmax);
+  IdT* wid = wid0 + (threadIdx.x >> 5) * (32 * GSS_CLS_U);                                      // per-warp id staging
+  uint32_t* lut = reinterpret_cast<uint32_t*>(wid0 + NW * (32 * GSS_CLS_U));                    // kLutN entries
+  uint32_t* s_scan = lut + kLutN;
   const Cmp less;
   const uint32_t slot = level & 1;
   const uint32_t nt = c.cnt->lvl[level].num_tiles;
@@ -450,6 +586,11 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
   // node j of levels 5..7 is read by this lane at rep_b + 128 j
   const uint32_t rep_b = (uint32_t)__cvta_generic_to_shared(rep) - (1u << kTopLevels) * 128u +
                          (threadIdx.x % REP) * (uint32_t)sizeof(Key);
+  // the radix-indexed lookup replaces the descent for unsigned keys under operator< (not for partition_by)
+  constexpr bool kLut = LUT && lut_ok<Key, Cmp>() && !PART;
+  ClsSrc<Key> cs;
+  cs.tree_s = tree_s; cs.rep_b = rep_b; cs.lut_s = (uint32_t)__cvta_generic_to_shared(lut);
+  cs.shift = 0; cs.base = Key(0); cs.logk = 0; cs.use_lut = false;
   uint32_t cur = 0xffffffffu;
   for (uint32_t t = t0; t < t1; t++) {
     const uint32_t b = c.tile_bucket[slot][t];
@@ -459,6 +600,7 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
       const Key* g = c.spl[slot] + B.spl_base;
       for (uint32_t j = threadIdx.x + 1; j < B.ks; j += kClsThreads) tree[j] = g[j];
       for (uint32_t j = threadIdx.x; j + 1 < B.ks; j += kClsThreads) spl[j] = g[B.kb + j];
+      if constexpr (kLut) cs.use_lut = lut_build(lut, spl, B.ks - 1, cs.base, cs.shift, s_scan);
       if (B.ks > (1u << kTopLevels)) {
         const uint32_t nrep = (min(B.ks, 1u << kRepEnd) - (1u << kTopLevels)) * REP;
         for (uint32_t q = threadIdx.x; q < nrep; q += kClsThreads) rep[q] = g[(1u << kTopLevels) + q / REP];
@@ -470,18 +612,21 @@ __global__ void __launch_bounds__(kClsThreads, GSS_CLS_MINB) k_classify(Ctx<Key,
     const uint32_t tl = t - B.tile_start;
     const uint32_t beg = B.lo + tl * c.T;
     const uint32_t len = min(c.T, B.m - tl * c.T);
-    const uint32_t logk = ilog2(B.ks);
+    cs.logk = ilog2(B.ks);
     IdT* tids = c.ids + B.id_base + tl * c.T;                  // 16-byte aligned per tile
     if constexpr (PART) {
-      if (B.eq) classify_tile<3, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
-      else classify_tile<2, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+      if (B.eq) classify_tile<3, true, false>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
+      else classify_tile<2, true, false>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
     } else if (c.recompute) {
-      if (B.eq) classify_tile<1, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
-      else classify_tile<0, false>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+      if (B.eq) classify_tile<1, false, kLut>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
+      else classify_tile<0, false, kLut>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
+    } else if constexpr (kLut) {
+      if (B.eq) classify_tile<1, true, true>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
+      else classify_tile<0, true, true>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
     } else if (B.eq) {
-      classify_tile<1, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+      classify_tile<1, true, false>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
     } else {
-      classify_tile<0, true>(src, tids, beg, len, tree_s, rep_b, spl, logk, B.ks, B.K, wc_s, wid, less);
+      classify_tile<0, true, false>(src, tids, beg, len, cs, spl, B.ks, B.K, wc_s, wid, less);
     }
     __syncthreads();
     uint32_t* hist = c.hist[slot] + B.hist_base;

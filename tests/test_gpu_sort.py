@@ -77,6 +77,68 @@ def test_partition_level_bit_exact(gss, oracle_mod, width, dist, with_vals):
 
 
 # ---------------------------------------------------------------------------
+# Phase 2 by the radix-indexed splitter lookup (default for unsigned keys)
+# against the paper's tree descent (GSS_FLAG_TREE_CLASSIFY = 512): both must
+# give the oracle's ids, so the stable partition is bit-exact either way.
+# Inputs aimed at the lookup's corners: keys at 0 and the type maximum, a
+# dense cluster that puts many splitters into one bin (the binary-search
+# path), a span of one or two key values (shift 0), the full 64-bit range
+# (shift 52), below-range keys (bin 0).
+# ---------------------------------------------------------------------------
+def _lut_case(case, n, width, seed=11):
+    rng = np.random.default_rng(seed)
+    dt = np.uint32 if width == 32 else np.uint64
+    mx = int(np.iinfo(dt).max)
+    if case == "extremes":
+        return rng.choice(np.array([0, 1, mx - 1, mx], dtype=dt), n)
+    if case == "cluster":
+        x = rng.integers(0, mx, n, dtype=dt, endpoint=True)
+        c = rng.integers(1 << (width - 8), (1 << (width - 8)) + 3000, n, dtype=dt)
+        return np.where(rng.random(n) < 0.9, c, x).astype(dt)
+    if case == "narrow":
+        return rng.integers(1 << (width - 2), (1 << (width - 2)) + 2, n, dtype=dt)
+    if case == "full":
+        x = rng.integers(0, mx, n, dtype=dt, endpoint=True)
+        x[::97] = 0
+        x[::89] = mx
+        return x
+    raise ValueError(case)
+
+
+LUT_CASES = ["extremes", "cluster", "narrow", "full"]
+
+
+@pytest.mark.parametrize("width", [32, 64])
+@pytest.mark.parametrize("case", LUT_CASES + ["uniform", "and4", "sorted"])
+@pytest.mark.parametrize("flags", [0, 512])
+def test_partition_lookup_vs_tree(gss, oracle_mod, width, case, flags):
+    n = 5 * 2048 * 3 + 777
+    x = _lut_case(case, n, width) if case in LUT_CASES else inputs.keys(case, n, width, seed=3)
+    for k in (16, 128, 1024):
+        prm = dict(k=k, a=30, seed=77, k_policy="fixed", tile=2048, flags=flags)
+        ko, _, spl, off, info = gss.partition(to_dev(x), None, **prm)
+        ok, _, rec = oracle_mod.distribute(x, None, oracle_params(oracle_mod, k=k, seed=77, k_policy="fixed", M=0))
+        assert info == (rec.kb, rec.ks, rec.eq, rec.K)
+        np.testing.assert_array_equal(to_host(off).astype(np.uint64),
+                                      np.concatenate([[0], np.cumsum(rec.children)]).astype(np.uint64))
+        np.testing.assert_array_equal(to_host(ko), ok)
+
+
+@pytest.mark.parametrize("width,pairs", [(32, False), (64, False), (64, True)])
+@pytest.mark.parametrize("case", LUT_CASES)
+def test_sort_lookup_corner_inputs(gss, oracle_mod, width, pairs, case):
+    n = (1 << 20) + 4321
+    x = _lut_case(case, n, width)
+    v = inputs.values(n, width) if pairs else None
+    ko, vo, st = gss.sort(to_dev(x), to_dev(v) if pairs else None, M=4096, stats=True)
+    ok, _, recs = oracle_mod.sort(x, None, oracle_params(oracle_mod, M=4096), log=True)
+    np.testing.assert_array_equal(to_host(ko), ok)
+    if pairs:
+        check_pairs(x, to_host(vo), ok)
+    assert_levels_match(st, recs)
+
+
+# ---------------------------------------------------------------------------
 # Whole sort: keys bit-exact vs the oracle, values as a multiset
 # ---------------------------------------------------------------------------
 KINDS = [(32, False), (64, False), (32, True), (64, True)]
@@ -627,7 +689,7 @@ def test_gss_hpp_user_comparators(gss, cxx_lib, n):
 # ---------------------------------------------------------------------------
 @pytest.mark.parametrize("width,pairs", KINDS)
 @pytest.mark.parametrize("variant", [dict(cls_arrays=1), dict(cls_arrays=2), dict(cls_arrays=4),
-                                     dict(flags=128), dict(flags=32), dict(flags=128 | 16)])
+                                     dict(flags=128), dict(flags=32), dict(flags=128 | 16), dict(flags=512)])
 def test_ablation_variants_vs_oracle(gss, oracle_mod, width, pairs, variant):
     n = (1 << 21) + 333
     x = inputs.keys("and3", n, width, seed=31)

@@ -40,6 +40,7 @@ def dem(n):
 target = None
 def norm(s):
     s = s.split("(gss::Ctx")[0]
+    s = s.replace("(bool)0", "false").replace("(bool)1", "true")
     return re.sub(r"\(int\)|\s+", "", s)
 kn = norm(kname)
 for f in funcs:
@@ -66,5 +67,5 @@ for r in data:
     agg[ln][0] += i; agg[ln][1] += s; ti += i; ts += s
 print(kname[:120])
 print(f"total warp-instructions {ti:.4g}, stall samples {ts:.4g}")
-for (f, l), (i, s) in sorted(agg.items(), key=lambda kv: -kv[1][1])[:top]:
+for (f, l), (i, s) in sorted(agg.items(), key=lambda kv: -kv[1][int(os.environ.get("LP_SORT_STALL", "1"))])[:top]:
     print(f"{f}:{l:<5d} inst {i/ti*100:5.1f}%  stall {s/ts*100:5.1f}%")
