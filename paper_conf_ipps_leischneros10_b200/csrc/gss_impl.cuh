@@ -37,6 +37,7 @@ namespace gssh {
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
 inline constexpr uint32_t kFlagScatterBulk = 1u << 29;          // ablation: bulk-copy scatter for 4-byte keys too
+inline constexpr uint32_t kFlagScatterNoWs = 1u << 27;          // ablation: the single-role bulk scatter (k_scatter_bulk)
 inline constexpr uint32_t kFlagSmallNarrow = 1u << 28;          // ablation: 48-register block sort for classes <= 20 warps
                                                                 // (2^28 u64: 4.98 vs 4.90 ms -- occupancy is not the limit)
 
@@ -395,6 +396,22 @@ struct Engine {
     const bool use_bulk = c.nremote || (!c.stable && !c.recompute && (bulk_default || (cfg.flags & kFlagScatterBulk)) &&
                           !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS)) &&
                           !((cfg.flags & kFlagScatterCtaCounters) && kHasVal<Val>));
+    // warp-specialised scatter: keys without values on the bulk path, local destinations, shared memory for
+    // two chunk buffers at this kmax (k <= 512)
+    bool use_ws = false;
+    auto kws = k_scatter_bulk<Key, Val, IdT, 1>;
+    size_t sm_ws = 0;
+    int g_ws = 0;
+    if constexpr (!kHasVal<Val>) {
+      sm_ws = ScatterWsSmem<Key, IdT>::bytes(kmax);
+      use_ws = use_bulk && !c.nremote && kmax <= 512 && sm_ws <= 113 * 1024 &&
+               !(cfg.flags & (kFlagScatterCtaCounters | kFlagScatterNoWs));
+      if (use_ws) {
+        kws = k_scatter_ws<Key, Val, IdT>;
+        GSS_TRY(set_smem(kws, sm_ws));
+        g_ws = grid_for(kws, kScatterThreads, sm_ws, di.sms);
+      }
+    }
     auto ksd = k_scatter_direct<Key, Val, IdT, Cmp>;
     const size_t sm_sd = (size_t)kmax * 4;
     GSS_TRY(set_smem(ksd, sm_sd));
@@ -416,7 +433,9 @@ struct Engine {
       // default and stable ranks (R7, GSS_FLAG_STABLE): k_scatter with per-warp counters (deterministic);
       // ablations: k_scatter_fast (one counter set per CTA: atomic order across warps is not
       // deterministic) and the paper's direct scatter (k_scatter_direct)
-      if (use_bulk) {
+      if (use_ws) {
+        GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { kws<<<g_ws, kScatterThreads, sm_ws, s>>>(c, l, kmax); }));
+      } else if (use_bulk) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksb<<<g_sb, kScatterThreads, sm_sb, s>>>(c, l, kmax); }));
       } else if (c.stable || !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | kFlagScatterCtaCounters))) {
         GSS_TRY(launch(prof, GSS_K_SCATTER, s, count, [&] { ksc<<<g_sc, kScatterThreads, sm_sc, s>>>(c, l, kmax); }));

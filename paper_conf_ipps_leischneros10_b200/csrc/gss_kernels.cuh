@@ -1358,7 +1358,11 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
       const uint32_t L = rlen[id];
       if (!L) continue;
       const uint32_t g = gbase[id], st = rstart[id];
-      if (!c.nremote) {
+#ifndef GSS_SCATTER_NOWRITE
+#define GSS_SCATTER_NOWRITE 0   // diagnostic (wrong output): the write phase skipped, to time everything else
+#endif
+      if (GSS_SCATTER_NOWRITE) {
+      } else if (!c.nremote) {
         put(kdst + g, kHasVal<Val> ? vdst + g : nullptr, st, L);
       } else {
         // fused exchange: the run goes to the GPUs owning its partition indices
@@ -1381,6 +1385,323 @@ __global__ void __launch_bounds__(kScatterThreads, GSS_SCATTER_MINB)
   if (c.nremote) __threadfence_system();                          // peer stores visible before the exchange barrier
 }
 
+// ---------------------------------------------------------------------------
+// Phase 4, warp-specialised (keys without values; the default for 8-byte
+// keys).  The single-role scatter (k_scatter_bulk) runs every phase of a chunk
+// in all 16 warps between CTA barriers; its write phase -- one warp-serialised
+// bulk copy per bucket run -- was a quarter of its instructions (ncu source
+// page, profiles/r02_*), and the global loads of the next chunk were exposed
+// at the top of every chunk.  Here warp 15 (the I/O warp) moves the data and
+// warps 0..14 (the rank warps) count and reorder:
+//  * the I/O warp loads each chunk (C = 15 x 256 keys and their ids) into
+//    shared memory by cp.async.bulk global -> shared, completing on an
+//    mbarrier (full[b], b = chunk parity); two chunk buffers, so chunk c+1 is
+//    in flight while chunk c is ranked;
+//  * the rank warps read their 8 keys per lane from the buffer, rank them on
+//    per-warp counters (one shared atomic per key; two ids share a 32-bit
+//    word, 16 bits each), fold and scan the counters among themselves (named
+//    barrier 1, 480 threads), and stage the chunk grouped by bucket id in the
+//    SAME buffer (every rank warp has read it before the first barrier), each
+//    key with its global destination index in a parallel array; then they
+//    arrive on named barrier 2+b without waiting;
+//  * the I/O warp syncs on 2+b and streams the staged chunk out in slot order,
+//    32 consecutive slots per store instruction (runs are contiguous, so the
+//    stores coalesce per bucket run), then loads chunk c+2 into the buffer.
+// Ranks within (warp, id) follow item order and the warps are folded in
+// order, so each level is a stable partition exactly as in k_scatter_bulk
+// (the oracle's level records hold).  GSS kFlagScatterNoWs: the single-role
+// kernel (ablation).
+// ---------------------------------------------------------------------------
+namespace wsync {
+__device__ __forceinline__ void bar_sync(uint32_t id, uint32_t n) {
+  asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(n) : "memory");
+}
+__device__ __forceinline__ void bar_arrive(uint32_t id, uint32_t n) {
+  asm volatile("bar.arrive %0, %1;" ::"r"(id), "r"(n) : "memory");
+}
+__device__ __forceinline__ void mbar_init(uint32_t a, uint32_t cnt) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(a), "r"(cnt) : "memory");
+}
+__device__ __forceinline__ void mbar_arrive_tx(uint32_t a, uint32_t tx) {
+  asm volatile("{\n\t.reg .b64 st;\n\tmbarrier.arrive.expect_tx.shared::cta.b64 st, [%0], %1;\n\t}" ::"r"(a), "r"(tx)
+               : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint32_t a, uint32_t parity) {
+  asm volatile(
+      "{\n\t.reg .pred p;\n\tLAB_WAIT:\n\t"
+      "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+      "@!p bra LAB_WAIT;\n\t}" ::"r"(a), "r"(parity)
+      : "memory");
+}
+__device__ __forceinline__ void bulk_g2s(uint32_t sdst, const void* gsrc, uint32_t bytes, uint32_t mbar) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(sdst),
+               "l"(gsrc), "r"(bytes), "r"(mbar)
+               : "memory");
+}
+}  // namespace wsync
+
+template <class Key, class IdT>
+struct ScatterWsSmem {
+  static constexpr uint32_t NR = kScatterThreads / 32 - 1;                 // rank warps
+  static constexpr uint32_t ITER = GSS_SCATTER_ITER;
+  static constexpr uint32_t C = NR * 32 * ITER;                            // keys per chunk
+  static constexpr uint32_t A = 16 / sizeof(Key);
+  static constexpr size_t buf_bytes() { return ((size_t)(C + A) * sizeof(Key) + 15) & ~size_t(15); }
+  static constexpr size_t dst_bytes() { return ((size_t)C * 4 + 15) & ~size_t(15); }
+  static constexpr size_t ids_bytes() { return ((size_t)C * sizeof(IdT) + 15) & ~size_t(15); }
+  // counters NR x kmax/2 words; gbase, delta: kmax each; scan 64 words; 2 mbarriers
+  __host__ __device__ static size_t head_bytes(uint32_t kmax) {
+    return ((size_t)NR * ((kmax + 1) / 2) + 2 * (size_t)kmax + 64) * 4 + 32;
+  }
+  __host__ __device__ static size_t bytes(uint32_t kmax) {
+    return 2 * (buf_bytes() + dst_bytes() + ids_bytes()) + ((head_bytes(kmax) + 15) & ~size_t(15));
+  }
+};
+
+template <class Key, class Val, class IdT>
+__global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+  static_assert(!kHasVal<Val>, "keys only");
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  using SM = ScatterWsSmem<Key, IdT>;
+  constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, NRT = NR * 32;
+  // per chunk parity b (selected arithmetically: no local-memory arrays)
+  constexpr size_t PB = SM::buf_bytes() + SM::dst_bytes() + SM::ids_bytes();
+  auto bufk = [&](uint32_t b) { return reinterpret_cast<Key*>(smem_raw + b * PB); };
+  auto bufd = [&](uint32_t b) { return reinterpret_cast<uint32_t*>(smem_raw + b * PB + SM::buf_bytes()); };
+  auto bufi = [&](uint32_t b) {
+    return reinterpret_cast<IdT*>(smem_raw + b * PB + SM::buf_bytes() + SM::dst_bytes());
+  };
+  const uint32_t KH = (kmax + 1) / 2;
+  uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw + 2 * PB);   // NR x KH packed counters, then offsets
+  uint32_t* gbase = cnt + NR * KH;                       // next global index of each id (owner threads)
+  uint32_t* delta = gbase + kmax;                        // this chunk: destination - staging slot of each id
+  uint32_t* s_warp = delta + kmax;                       // 64 words
+  const uint32_t mbar_0 = ((uint32_t)__cvta_generic_to_shared(s_warp + 64) + 7) & ~7u;
+  auto mbar = [&](uint32_t b) { return mbar_0 + 8 * b; };
+
+  const uint32_t slot = level & 1;
+  const uint32_t nt = c.cnt->lvl[level].num_tiles;
+  const Key* ksrc = c.keys(c.src(level));
+  Key* kdst = c.wkeys(c.dst(level));
+  const IdT* idsrc = c.ids;
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  if (blockIdx.x >= nt) return;
+  if (threadIdx.x == 0) {
+    wsync::mbar_init(mbar(0), 1);
+    wsync::mbar_init(mbar(1), 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+
+  // The chunk sequence of this CTA: tiles blockIdx.x, +gridDim.x, ...; chunks of C keys inside each tile.
+  struct Cursor {
+    uint32_t t, c0, beg, len, K, idb;
+    bool valid;
+  };
+  auto tile_at = [&](Cursor& u) {
+    const Bucket B = c.bk[slot][c.tile_bucket[slot][u.t]];
+    const uint32_t tl = u.t - B.tile_start;
+    u.beg = B.lo + tl * c.T;
+    u.len = min(c.T, B.m - tl * c.T);
+    u.K = B.K;
+    u.idb = B.id_base + tl * c.T;
+  };
+  auto advance = [&](Cursor& u) {                        // new tile: u.c0 == 0
+    u.c0 += C;
+    if (u.c0 >= u.len) {
+      u.t += gridDim.x;
+      u.c0 = 0;
+      u.valid = u.t < nt;
+      if (u.valid) tile_at(u);
+    }
+  };
+  Cursor cur;
+  cur.t = blockIdx.x; cur.c0 = 0; cur.valid = true;
+  tile_at(cur);
+
+  if (w == (int)NR) {
+    // ------------------------------ I/O warp ------------------------------
+    auto load = [&](const Cursor& u, uint32_t b) {
+      const uint32_t clen = min(C, u.len - u.c0);
+      const uint32_t g0 = u.beg + u.c0;
+      const uint32_t sh = g0 & (A - 1);                  // element q lives in slot q + sh (16-byte phase of g0)
+      const uint32_t h = min(clen, (A - sh) & (A - 1));  // head elements before the aligned middle
+      const uint32_t mid = (clen - h) & ~(A - 1);
+      const uint32_t ib = (clen * (uint32_t)sizeof(IdT)) & ~15u;   // id bytes by bulk copy (16-byte aligned start)
+      Key* bk = bufk(b);
+      IdT* bi = bufi(b);
+      for (uint32_t q = lane; q < h; q += 32) bk[q + sh] = ksrc[g0 + q];
+      for (uint32_t q = h + mid + lane; q < clen; q += 32) bk[q + sh] = ksrc[g0 + q];
+      for (uint32_t q = ib / (uint32_t)sizeof(IdT) + lane; q < clen; q += 32) bi[q] = idsrc[u.idb + u.c0 + q];
+      __syncwarp();
+      if (lane == 0) {
+        fence_proxy_async_smem();                        // the buffer's generic accesses before the async writes
+        wsync::mbar_arrive_tx(mbar(b), mid * (uint32_t)sizeof(Key) + ib);
+        if (mid)
+          wsync::bulk_g2s((uint32_t)__cvta_generic_to_shared(bk + h + sh), ksrc + g0 + h, mid * (uint32_t)sizeof(Key),
+                          mbar(b));
+        if (ib) wsync::bulk_g2s((uint32_t)__cvta_generic_to_shared(bi), idsrc + u.idb + u.c0, ib, mbar(b));
+      }
+    };
+    Cursor ld = cur;                                     // load cursor: two chunks ahead of the stores
+    load(ld, 0);
+    advance(ld);
+    if (ld.valid) load(ld, 1);
+    for (uint32_t k = 0;; k++) {
+      const uint32_t b = k & 1;
+      const uint32_t clen = min(C, cur.len - cur.c0);
+      wsync::bar_sync(2 + b, kScatterThreads);           // chunk k staged in buffer b
+      const Key* stg = bufk(b);
+      const uint32_t* dd = bufd(b);
+      // the staged chunk in slot order: 32 consecutive slots per store, four stores in flight per lane
+      uint32_t s = lane;
+      for (; s + 96 < clen; s += 128) {
+        Key x[4];
+        uint32_t y[4];
+#pragma unroll
+        for (int u = 0; u < 4; u++) { x[u] = stg[s + 32 * u]; y[u] = dd[s + 32 * u]; }
+#pragma unroll
+        for (int u = 0; u < 4; u++) kdst[y[u]] = x[u];
+      }
+      for (; s < clen; s += 32) kdst[dd[s]] = stg[s];
+      advance(cur);
+      if (ld.valid) advance(ld);
+      __syncwarp();
+      if (ld.valid) load(ld, b);                         // chunk k+2 into buffer b
+      if (!cur.valid) break;
+    }
+    return;
+  }
+
+  // ------------------------------ rank warps ------------------------------
+  const uint32_t* wc = cnt + w * KH;
+  const uint32_t wc_s = (uint32_t)__cvta_generic_to_shared(wc);
+  const uint32_t own = threadIdx.x;                      // owner of ids 2*own, 2*own+1
+  for (uint32_t k = 0;; k++) {
+    const uint32_t b = k & 1;
+    const uint32_t K = cur.K, KP = (K + 1) / 2;
+    if (cur.c0 == 0 && own < KP) {                       // a new tile: the global start of each id in it
+      const Bucket B = c.bk[slot][c.tile_bucket[slot][cur.t]];
+      const uint32_t tl = cur.t - B.tile_start;
+      const uint32_t* hist = c.hist[slot] + B.hist_base;
+      const uint32_t hb = hist[0];
+#pragma unroll
+      for (uint32_t j = 0; j < 2; j++) {
+        const uint32_t id = 2 * own + j;
+        if (id < K) gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
+      }
+    }
+    const uint32_t clen = min(C, cur.len - cur.c0);
+    const uint32_t sh = (cur.beg + cur.c0) & (A - 1);
+    for (uint32_t j = lane; j < KP; j += 32) cnt[w * KH + j] = 0;
+    wsync::mbar_wait(mbar(b), (k >> 1) & 1);
+    Key kk[ITER];
+    uint32_t iid[ITER];
+    const Key* bk = bufk(b);
+    const IdT* bi = bufi(b);
+#pragma unroll
+    for (uint32_t it = 0; it < ITER; it++) {
+      const uint32_t q = w * (32 * ITER) + it * 32 + lane;
+      iid[it] = 0xffffffffu;
+      if (q < clen) {
+        kk[it] = bk[q + sh];
+        iid[it] = bi[q];
+      }
+    }
+    __syncwarp();
+    // ranks within (warp, id): packed counters, two ids per word
+    {
+      const uint32_t first = __shfl_sync(kFull, iid[0], 0);
+      bool same = first != 0xffffffffu;
+#pragma unroll
+      for (uint32_t it = 0; it < ITER; it++) same = same && iid[it] == first;
+      if (__all_sync(kFull, same)) {
+        uint32_t base = 0;
+        if (lane == 0) base = atom_add_shared_if(1u, wc_s + 4 * (first >> 1), (32u * ITER) << (16 * (first & 1)));
+        base = (__shfl_sync(kFull, base, 0) >> (16 * (first & 1))) & 0xffffu;
+#pragma unroll
+        for (uint32_t it = 0; it < ITER; it++) iid[it] = ((base + 32u * it + (uint32_t)lane) << 16) | first;
+      } else {
+#pragma unroll
+        for (uint32_t it = 0; it < ITER; it++) {
+          const uint32_t id = iid[it] & 0xffffu, hs = 16 * (id & 1);
+          const uint32_t r = atom_add_shared_if(iid[it] != 0xffffffffu ? 1u : 0u, wc_s + 4 * (id >> 1), 1u << hs);
+          iid[it] = iid[it] == 0xffffffffu ? iid[it] : (((r >> hs) & 0xffffu) << 16) | id;
+        }
+      }
+    }
+    wsync::bar_sync(1, NRT);                             // counters complete; every rank warp has read buffer b
+    // owners: chunk totals of ids 2*own, 2*own+1 (runs packed in id order), every warp's start in them
+    uint32_t L0 = 0, L1 = 0;
+    if (own < KP) {
+#pragma unroll
+      for (uint32_t q = 0; q < NR; q++) {
+        const uint32_t x = cnt[q * KH + own];
+        L0 += x & 0xffffu;
+        L1 += x >> 16;
+      }
+    }
+    const uint32_t tsum = L0 + L1;                       // an odd K's missing id counts 0
+    uint32_t ex;
+    {
+      uint32_t inc = tsum;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(kFull, inc, o);
+        if (lane >= o) inc += y;
+      }
+      if (lane == 31) s_warp[w] = inc;
+      wsync::bar_sync(1, NRT);
+      if (w == 0) {
+        const uint32_t v = lane < (int)NR ? s_warp[lane] : 0u;
+        uint32_t vi = v;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+          const uint32_t y = __shfl_up_sync(kFull, vi, o);
+          if (lane >= o) vi += y;
+        }
+        if (lane < (int)NR) s_warp[32 + lane] = vi - v;
+      }
+      wsync::bar_sync(1, NRT);
+      ex = s_warp[32 + w] + inc - tsum;
+    }
+    if (own < KP) {
+      const uint32_t st0 = ex, st1 = ex + L0;
+      const uint32_t id0 = 2 * own;
+      delta[id0] = gbase[id0] - st0;
+      gbase[id0] += L0;
+      if (id0 + 1 < K) {
+        delta[id0 + 1] = gbase[id0 + 1] - st1;
+        gbase[id0 + 1] += L1;
+      }
+      uint32_t r0 = st0, r1 = st1;
+#pragma unroll
+      for (uint32_t q = 0; q < NR; q++) {
+        const uint32_t x = cnt[q * KH + own];
+        cnt[q * KH + own] = r0 | (r1 << 16);
+        r0 += x & 0xffffu;
+        r1 += x >> 16;
+      }
+    }
+    wsync::bar_sync(1, NRT);                             // run slots known
+    Key* sk = bufk(b);
+    uint32_t* sd = bufd(b);
+#pragma unroll
+    for (uint32_t it = 0; it < ITER; it++) {
+      if (iid[it] != 0xffffffffu) {
+        const uint32_t id = iid[it] & 0xffffu;
+        const uint32_t pos = ((wc[id >> 1] >> (16 * (id & 1))) & 0xffffu) + (iid[it] >> 16);
+        sk[pos] = kk[it];
+        sd[pos] = pos + delta[id];
+      }
+    }
+    wsync::bar_arrive(2 + b, kScatterThreads);
+    advance(cur);
+    if (!cur.valid) break;
+  }
+}
+
+// ---------------------------------------------------------------------------
 // Phase 4, default variant (R7: a partition, not stable).  Every key takes
 // its rank within (chunk, id) from one shared-memory atomic on the CTA's
 // counter for its id; warp 0 scans the K chunk totals into staged run
