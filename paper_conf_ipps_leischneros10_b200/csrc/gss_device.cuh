@@ -251,6 +251,10 @@ __device__ __forceinline__ uint64_t block_sum_u64(uint64_t x, unsigned long long
 __host__ __device__ constexpr int padded_len(int c) { return (c + c / 16 + 1 + 3) & ~3; }
 __device__ __forceinline__ int phys(int i) { return i + (i >> 4); }
 
+#ifndef GSS_SEARCH_UNROLL
+#define GSS_SEARCH_UNROLL 2   // merge-path search steps per loop iteration
+#endif
+constexpr int kSearchUnroll = GSS_SEARCH_UNROLL;
 #ifndef GSS_FAST_KV
 #define GSS_FAST_KV 0      // 1: PTX merge step for key-value pairs (measured slower: 4.69 vs 4.57 ms, 2^27 u64 pairs)
 #endif
@@ -619,6 +623,7 @@ struct CtaSort {
 #if GSS_SEARCH_CLZ
       for (int st = hi > lo ? 1 << (31 - __clz(hi - lo)) : 0; st > 0; st >>= 1) {
 #else
+#pragma unroll kSearchUnroll
       for (int st = w; st > 0; st >>= 1) {
 #endif
         const int pr = j + st - 1;
@@ -637,6 +642,7 @@ struct CtaSort {
 #if GSS_SEARCH_CLZ
       for (int st = hi > lo ? 1 << (31 - __clz(hi - lo)) : 0; st > 0; st >>= 1) {
 #else
+#pragma unroll kSearchUnroll
       for (int st = w; st > 0; st >>= 1) {
 #endif
         const int pr = j + st - 1;
@@ -851,7 +857,10 @@ struct CtaSort {
     // only synchronise the warp; wider rounds synchronise the block.
     for (int w = w0; w < m; w *= 2) {
       const bool blk = NT > 32 && nt > 32 && 2 * w > 32 * ITEMS;
-      if (blk) __syncthreads(); else __syncwarp();
+      auto round_bar = [&]() {
+        if (blk) __syncthreads(); else __syncwarp();
+      };
+      round_bar();
       const int ps = base & ~(2 * w - 1);                // w is a power of two
       const int aLen = min(w, m - ps);
       const int bLen = max(0, min(w, m - ps - w));
@@ -868,7 +877,7 @@ struct CtaSort {
           }
         }
       }
-      if (blk) __syncthreads(); else __syncwarp();
+      round_bar();
       if (cnt > 0) store_run(sk, sv, k, v, cnt, ps, aLen + bLen, base - ps, (base & (2 * w)) != 0);
     }
     bar(nt);
