@@ -1440,22 +1440,24 @@ __device__ __forceinline__ void bulk_g2s(uint32_t sdst, const void* gsrc, uint32
 }
 }  // namespace wsync
 
+#ifndef GSS_SCATTER_IO_WARPS
+#define GSS_SCATTER_IO_WARPS 2   // one I/O warp could not keep up with the stores (rank warps waited on it)
+#endif
 template <class Key, class IdT>
 struct ScatterWsSmem {
-  static constexpr uint32_t NR = kScatterThreads / 32 - 1;                 // rank warps
+  static constexpr uint32_t NIO = GSS_SCATTER_IO_WARPS;                    // I/O warps
+  static constexpr uint32_t NR = kScatterThreads / 32 - NIO;               // rank warps
   static constexpr uint32_t ITER = GSS_SCATTER_ITER;
   static constexpr uint32_t C = NR * 32 * ITER;                            // keys per chunk
   static constexpr uint32_t A = 16 / sizeof(Key);
-  static constexpr size_t buf_bytes() { return ((size_t)(C + A) * sizeof(Key) + 15) & ~size_t(15); }
-  static constexpr size_t dst_bytes() { return ((size_t)C * 4 + 15) & ~size_t(15); }
-  static constexpr size_t ids_bytes() { return ((size_t)C * sizeof(IdT) + 15) & ~size_t(15); }
-  // counters NR x kmax/2 words; gbase, delta: kmax each; scan 64 words; 2 mbarriers
+  static constexpr size_t al(size_t x) { return (x + 15) & ~size_t(15); }
+  static constexpr size_t in_bytes() { return al((size_t)(C + A) * sizeof(Key)) + al((size_t)C * sizeof(IdT)); }
+  static constexpr size_t stage_bytes() { return al((size_t)C * sizeof(Key)) + al((size_t)C * sizeof(IdT)); }
+  // counters NR x kmax/2 words; gbase kmax; delta 2 x kmax; scan 64 words; 2 mbarriers
   __host__ __device__ static size_t head_bytes(uint32_t kmax) {
-    return ((size_t)NR * ((kmax + 1) / 2) + 2 * (size_t)kmax + 64) * 4 + 32;
+    return al(((size_t)NR * ((kmax + 1) / 2) + 3 * (size_t)kmax + 64) * 4 + 32);
   }
-  __host__ __device__ static size_t bytes(uint32_t kmax) {
-    return 2 * (buf_bytes() + dst_bytes() + ids_bytes()) + ((head_bytes(kmax) + 15) & ~size_t(15));
-  }
+  __host__ __device__ static size_t bytes(uint32_t kmax) { return 2 * in_bytes() + stage_bytes() + head_bytes(kmax); }
 };
 
 template <class Key, class Val, class IdT>
@@ -1463,19 +1465,22 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
   static_assert(!kHasVal<Val>, "keys only");
   extern __shared__ __align__(16) unsigned char smem_raw[];
   using SM = ScatterWsSmem<Key, IdT>;
-  constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, NRT = NR * 32;
-  // per chunk parity b (selected arithmetically: no local-memory arrays)
-  constexpr size_t PB = SM::buf_bytes() + SM::dst_bytes() + SM::ids_bytes();
-  auto bufk = [&](uint32_t b) { return reinterpret_cast<Key*>(smem_raw + b * PB); };
-  auto bufd = [&](uint32_t b) { return reinterpret_cast<uint32_t*>(smem_raw + b * PB + SM::buf_bytes()); };
-  auto bufi = [&](uint32_t b) {
-    return reinterpret_cast<IdT*>(smem_raw + b * PB + SM::buf_bytes() + SM::dst_bytes());
+  constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, NRT = NR * 32, NIOT = SM::NIO * 32;
+  // named barriers: 1 the rank warps; 2 staged (rank warps arrive, I/O syncs); 3 staging free (I/O arrives,
+  // rank warps sync); 4+b input buffer b read (rank warps arrive, I/O syncs)
+  constexpr uint32_t BAR_RANK = 1, BAR_STAGED = 2, BAR_FREE = 3, BAR_IN = 4;
+  // input buffer b (selected arithmetically: no local-memory arrays)
+  auto ink = [&](uint32_t b) { return reinterpret_cast<Key*>(smem_raw + b * SM::in_bytes()); };
+  auto ini = [&](uint32_t b) {
+    return reinterpret_cast<IdT*>(smem_raw + b * SM::in_bytes() + SM::al((size_t)(C + A) * sizeof(Key)));
   };
+  Key* stk = reinterpret_cast<Key*>(smem_raw + 2 * SM::in_bytes());
+  IdT* sti = reinterpret_cast<IdT*>(smem_raw + 2 * SM::in_bytes() + SM::al((size_t)C * sizeof(Key)));
   const uint32_t KH = (kmax + 1) / 2;
-  uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw + 2 * PB);   // NR x KH packed counters, then offsets
+  uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw + 2 * SM::in_bytes() + SM::stage_bytes());
   uint32_t* gbase = cnt + NR * KH;                       // next global index of each id (owner threads)
-  uint32_t* delta = gbase + kmax;                        // this chunk: destination - staging slot of each id
-  uint32_t* s_warp = delta + kmax;                       // 64 words
+  uint32_t* delta = gbase + kmax;                        // per chunk parity: destination - staging slot of each id
+  uint32_t* s_warp = delta + 2 * kmax;                   // 64 words
   const uint32_t mbar_0 = ((uint32_t)__cvta_generic_to_shared(s_warp + 64) + 7) & ~7u;
   auto mbar = [&](uint32_t b) { return mbar_0 + 8 * b; };
 
@@ -1519,8 +1524,11 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
   cur.t = blockIdx.x; cur.c0 = 0; cur.valid = true;
   tile_at(cur);
 
-  if (w == (int)NR) {
-    // ------------------------------ I/O warp ------------------------------
+  if (w >= (int)NR) {
+    // ------------------------------ I/O warps ------------------------------
+    // warp NR loads; every I/O thread stores (slot io, io + NIOT, ...)
+    const uint32_t io = threadIdx.x - NRT;
+    const bool loader = w == (int)NR;
     auto load = [&](const Cursor& u, uint32_t b) {
       const uint32_t clen = min(C, u.len - u.c0);
       const uint32_t g0 = u.beg + u.c0;
@@ -1528,8 +1536,8 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
       const uint32_t h = min(clen, (A - sh) & (A - 1));  // head elements before the aligned middle
       const uint32_t mid = (clen - h) & ~(A - 1);
       const uint32_t ib = (clen * (uint32_t)sizeof(IdT)) & ~15u;   // id bytes by bulk copy (16-byte aligned start)
-      Key* bk = bufk(b);
-      IdT* bi = bufi(b);
+      Key* bk = ink(b);
+      IdT* bi = ini(b);
       for (uint32_t q = lane; q < h; q += 32) bk[q + sh] = ksrc[g0 + q];
       for (uint32_t q = h + mid + lane; q < clen; q += 32) bk[q + sh] = ksrc[g0 + q];
       for (uint32_t q = ib / (uint32_t)sizeof(IdT) + lane; q < clen; q += 32) bi[q] = idsrc[u.idb + u.c0 + q];
@@ -1543,31 +1551,32 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         if (ib) wsync::bulk_g2s((uint32_t)__cvta_generic_to_shared(bi), idsrc + u.idb + u.c0, ib, mbar(b));
       }
     };
-    Cursor ld = cur;                                     // load cursor: two chunks ahead of the stores
-    load(ld, 0);
+    Cursor ld = cur;                                     // load cursor: two chunks ahead
+    if (loader) load(ld, 0);
     advance(ld);
-    if (ld.valid) load(ld, 1);
+    if (ld.valid && loader) load(ld, 1);
     for (uint32_t k = 0;; k++) {
       const uint32_t b = k & 1;
       const uint32_t clen = min(C, cur.len - cur.c0);
-      wsync::bar_sync(2 + b, kScatterThreads);           // chunk k staged in buffer b
-      const Key* stg = bufk(b);
-      const uint32_t* dd = bufd(b);
-      // the staged chunk in slot order: 32 consecutive slots per store, four stores in flight per lane
-      uint32_t s = lane;
-      for (; s + 96 < clen; s += 128) {
+      wsync::bar_sync(BAR_IN + b, kScatterThreads);      // the rank warps have read input buffer b (chunk k)
+      if (ld.valid) advance(ld);
+      if (ld.valid && loader) load(ld, b);               // chunk k+2
+      wsync::bar_sync(BAR_STAGED, kScatterThreads);      // chunk k staged
+      // the staged chunk in slot order: 32 consecutive slots per store (runs are contiguous), four in flight
+      const uint32_t* dl = delta + b * kmax;
+      uint32_t s = io;
+      for (; s + 3 * NIOT < clen; s += 4 * NIOT) {
         Key x[4];
         uint32_t y[4];
 #pragma unroll
-        for (int u = 0; u < 4; u++) { x[u] = stg[s + 32 * u]; y[u] = dd[s + 32 * u]; }
+        for (int u = 0; u < 4; u++) { x[u] = stk[s + NIOT * u]; y[u] = s + NIOT * u + dl[sti[s + NIOT * u]]; }
 #pragma unroll
         for (int u = 0; u < 4; u++) kdst[y[u]] = x[u];
       }
-      for (; s < clen; s += 32) kdst[dd[s]] = stg[s];
-      advance(cur);
-      if (ld.valid) advance(ld);
+      for (; s < clen; s += NIOT) kdst[s + dl[sti[s]]] = stk[s];
       __syncwarp();
-      if (ld.valid) load(ld, b);                         // chunk k+2 into buffer b
+      wsync::bar_arrive(BAR_FREE, kScatterThreads);      // the staging buffer may be rewritten
+      advance(cur);
       if (!cur.valid) break;
     }
     return;
@@ -1597,18 +1606,21 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
     wsync::mbar_wait(mbar(b), (k >> 1) & 1);
     Key kk[ITER];
     uint32_t iid[ITER];
-    const Key* bk = bufk(b);
-    const IdT* bi = bufi(b);
+    {
+      const Key* bk = ink(b);
+      const IdT* bi = ini(b);
 #pragma unroll
-    for (uint32_t it = 0; it < ITER; it++) {
-      const uint32_t q = w * (32 * ITER) + it * 32 + lane;
-      iid[it] = 0xffffffffu;
-      if (q < clen) {
-        kk[it] = bk[q + sh];
-        iid[it] = bi[q];
+      for (uint32_t it = 0; it < ITER; it++) {
+        const uint32_t q = w * (32 * ITER) + it * 32 + lane;
+        iid[it] = 0xffffffffu;
+        if (q < clen) {
+          kk[it] = bk[q + sh];
+          iid[it] = bi[q];
+        }
       }
     }
     __syncwarp();
+    wsync::bar_arrive(BAR_IN + b, kScatterThreads);      // input buffer b may be refilled
     // ranks within (warp, id): packed counters, two ids per word
     {
       const uint32_t first = __shfl_sync(kFull, iid[0], 0);
@@ -1630,7 +1642,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         }
       }
     }
-    wsync::bar_sync(1, NRT);                             // counters complete; every rank warp has read buffer b
+    wsync::bar_sync(BAR_RANK, NRT);                      // counters complete
     // owners: chunk totals of ids 2*own, 2*own+1 (runs packed in id order), every warp's start in them
     uint32_t L0 = 0, L1 = 0;
     if (own < KP) {
@@ -1651,7 +1663,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         if (lane >= o) inc += y;
       }
       if (lane == 31) s_warp[w] = inc;
-      wsync::bar_sync(1, NRT);
+      wsync::bar_sync(BAR_RANK, NRT);
       if (w == 0) {
         const uint32_t v = lane < (int)NR ? s_warp[lane] : 0u;
         uint32_t vi = v;
@@ -1662,16 +1674,17 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         }
         if (lane < (int)NR) s_warp[32 + lane] = vi - v;
       }
-      wsync::bar_sync(1, NRT);
+      wsync::bar_sync(BAR_RANK, NRT);
       ex = s_warp[32 + w] + inc - tsum;
     }
     if (own < KP) {
+      uint32_t* dl = delta + b * kmax;
       const uint32_t st0 = ex, st1 = ex + L0;
       const uint32_t id0 = 2 * own;
-      delta[id0] = gbase[id0] - st0;
+      dl[id0] = gbase[id0] - st0;
       gbase[id0] += L0;
       if (id0 + 1 < K) {
-        delta[id0 + 1] = gbase[id0 + 1] - st1;
+        dl[id0 + 1] = gbase[id0 + 1] - st1;
         gbase[id0 + 1] += L1;
       }
       uint32_t r0 = st0, r1 = st1;
@@ -1683,22 +1696,22 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         r1 += x >> 16;
       }
     }
-    wsync::bar_sync(1, NRT);                             // run slots known
-    Key* sk = bufk(b);
-    uint32_t* sd = bufd(b);
+    if (k > 0) wsync::bar_sync(BAR_FREE, kScatterThreads);   // the I/O warp has written chunk k-1 out
+    wsync::bar_sync(BAR_RANK, NRT);                      // run slots known
 #pragma unroll
     for (uint32_t it = 0; it < ITER; it++) {
       if (iid[it] != 0xffffffffu) {
         const uint32_t id = iid[it] & 0xffffu;
         const uint32_t pos = ((wc[id >> 1] >> (16 * (id & 1))) & 0xffffu) + (iid[it] >> 16);
-        sk[pos] = kk[it];
-        sd[pos] = pos + delta[id];
+        stk[pos] = kk[it];
+        sti[pos] = (IdT)id;
       }
     }
-    wsync::bar_arrive(2 + b, kScatterThreads);
+    wsync::bar_arrive(BAR_STAGED, kScatterThreads);
     advance(cur);
     if (!cur.valid) break;
   }
+  wsync::bar_sync(BAR_FREE, kScatterThreads);            // matches the I/O warp's last arrival
 }
 
 // ---------------------------------------------------------------------------
