@@ -766,7 +766,12 @@ struct CtaSort {
 #endif
   static constexpr bool WB = GSS_WARP_BITONIC && !KV && BitwiseOrder<Cmp>::value && !BITONIC;
 
-  __device__ static void sort(Key* sk, Val* sv, int m, Cmp less, int nt = NT) {
+  // gk / gv (optional): the m keys (values) are read from global memory straight into the threads'
+  // registers instead of from sk / sv: thread t < m / ITEMS takes items t, t + m/ITEMS, t + 2 m/ITEMS, ...
+  // (every load instruction coalesced across the warp), the remainder goes to thread m / ITEMS.  Which keys
+  // a thread starts with is immaterial (it sorts them); the runs keep the layout of the shared-memory path.
+  __device__ static void sort(Key* sk, Val* sv, int m, Cmp less, int nt = NT, const Key* gk = nullptr,
+                              const Val* gv = nullptr) {
     bar(nt);
     const int t = NT == 32 ? (threadIdx.x & 31) : threadIdx.x;
     const int base = t * ITEMS;
@@ -808,11 +813,23 @@ struct CtaSort {
       }
       w0 = 32 * ITEMS;
     } else if (cnt > 0) {
+      if (gk) {
+        const int nf = m / ITEMS;                          // full threads
+        const int g0 = t < nf ? t : nf * ITEMS, gs = t < nf ? nf : 1;
 #pragma unroll
-      for (int i = 0; i < ITEMS; i++) {
-        if (i < cnt) {
-          k[i] = sk[phys(base + i)];
-          if constexpr (KV) v[i] = sv[phys(base + i)];
+        for (int i = 0; i < ITEMS; i++) {
+          if (i < cnt) {
+            k[i] = gk[g0 + i * gs];
+            if constexpr (KV) v[i] = gv[g0 + i * gs];
+          }
+        }
+      } else {
+#pragma unroll
+        for (int i = 0; i < ITEMS; i++) {
+          if (i < cnt) {
+            k[i] = sk[phys(base + i)];
+            if constexpr (KV) v[i] = sv[phys(base + i)];
+          }
         }
       }
       // A partial thread pads with copies of its largest item: after sorting,

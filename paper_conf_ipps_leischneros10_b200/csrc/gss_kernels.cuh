@@ -2206,6 +2206,10 @@ __host__ __device__ constexpr size_t block_sort_smem_bytes(int nt) {
   return (size_t)padded_len(nt * small_items<Key, Val>()) * (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0));
 }
 
+#ifndef GSS_SMALL_DIRECT
+#define GSS_SMALL_DIRECT 1   // bucket keys read by the sorting threads straight into registers: 2^27 u32 in-SM
+#endif                       // sort 1.61 -> 1.52 ms, u64 pairs 4.47 -> 4.33, u32 pairs 2.63 -> 2.56; 8-byte keys
+                             // alone keep the cp.async staging (4.76 vs 4.83 ms)
 #ifndef GSS_SMALL_CPASYNC
 #define GSS_SMALL_CPASYNC 1   // 8-byte keys: 4.83 vs 4.96 ms (2^28 u64), pairs 4.45 vs 4.57; 4-byte copies lose (2.15 vs 1.58)
 #endif
@@ -2232,6 +2236,10 @@ __global__ void __launch_bounds__(MAXT, MAXT <= kSmallNarrowThreads ? 2 : 1)
     const Key* src = c.keys(I.buf) + I.lo;
     const Val* vs = nullptr;
     if constexpr (kHasVal<Val>) vs = c.vals(I.buf) + I.lo;
+    if constexpr (GSS_SMALL_DIRECT && !Sorter::WB && !(sizeof(Key) == 8 && !kHasVal<Val>)) {
+      // the threads read their first items straight from global memory (no shared-memory staging)
+      Sorter::sort(sk, sv, (int)m, less, nt, src, vs);
+    } else {
     if constexpr (GSS_SMALL_CPASYNC && sizeof(Key) == 8) {
     // the bucket goes global -> shared by asynchronous copies (no registers,
     // every copy of the thread in flight at once)
@@ -2268,6 +2276,7 @@ __global__ void __launch_bounds__(MAXT, MAXT <= kSmallNarrowThreads ? 2 : 1)
     }
     }
     Sorter::sort(sk, sv, (int)m, less, nt);
+    }
     for (uint32_t q = threadIdx.x; q < m; q += nt) c.kout[I.lo + q] = sk[phys(q)];
     if constexpr (kHasVal<Val>)
       for (uint32_t q = threadIdx.x; q < m; q += nt) c.vout[I.lo + q] = sv[phys(q)];

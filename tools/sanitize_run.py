@@ -23,7 +23,8 @@ def run():
     for width in (32, 64):
         for pairs in (False, True):
             for dist, flags, extra in (("uniform", 0, {}), ("dd", 0, {}), ("and3", 4, {}), ("uniform", 8, {}),
-                                       ("staggered", 1, {}), ("uniform", 0, dict(max_levels=1, k=8, k_policy="fixed"))):
+                                       ("staggered", 1, {}), ("uniform", 0, dict(max_levels=1, k=8, k_policy="fixed")),
+                                       ("and4", 512, {}), ("sorted", 0, {})):
                 x = inputs.keys(dist, n, width, seed=3)
                 v = inputs.values(n, width) if pairs else None
                 kd = torch.from_numpy(x).cuda()
