@@ -403,11 +403,20 @@ struct Engine {
     size_t sm_ws = 0;
     int g_ws = 0;
     if constexpr (!kHasVal<Val>) {
-      sm_ws = ScatterWsSmem<Key, IdT>::bytes(kmax);
-      use_ws = use_bulk && !c.nremote && kmax <= 512 && sm_ws <= 113 * 1024 &&
-               !(cfg.flags & (kFlagScatterCtaCounters | kFlagScatterNoWs));
-      if (use_ws) {
+      // 14 rank + 2 I/O warps; where their chunk buffers do not fit two CTAs per SM (k = 512, 16-bit ids),
+      // 12 + 4 (shorter chunks)
+      constexpr size_t kWsMax = 113 * 1024;
+      const bool ok = use_bulk && !c.nremote && kmax <= 512 && !(cfg.flags & (kFlagScatterCtaCounters | kFlagScatterNoWs));
+      if (ok && ScatterWsSmem<Key, IdT>::bytes(kmax) <= kWsMax) {
+        use_ws = true;
+        sm_ws = ScatterWsSmem<Key, IdT>::bytes(kmax);
         kws = k_scatter_ws<Key, Val, IdT>;
+      } else if (ok && ScatterWsSmem<Key, IdT, 4>::bytes(kmax) <= kWsMax) {
+        use_ws = true;
+        sm_ws = ScatterWsSmem<Key, IdT, 4>::bytes(kmax);
+        kws = k_scatter_ws<Key, Val, IdT, 4>;
+      }
+      if (use_ws) {
         GSS_TRY(set_smem(kws, sm_ws));
         g_ws = grid_for(kws, kScatterThreads, sm_ws, di.sms);
       }

@@ -471,6 +471,9 @@ struct ClsSrc {
 // the warp stages its 256 ids in shared memory and writes them as one 8-byte
 // store per lane.  Full groups run without bounds tests; the next group's
 // keys are loaded before this group descends.
+#ifndef GSS_CLS_L2PF
+#define GSS_CLS_L2PF 3   // groups ahead of the L2 prefetch in Phase 2 (0: none)
+#endif
 template <int MODE, bool STORE, bool LUT, class Key, class IdT, class Cmp>
 __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* __restrict__ tids, uint32_t beg,
                                               uint32_t len, const ClsSrc<Key>& cs, const Key* spl,
@@ -502,6 +505,13 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
 #pragma unroll
       for (int u = 0; u < U; u++) nx[u] = sp[(g + 1) * G + u * 32];
     }
+#if GSS_CLS_L2PF
+    // the warp's keys of group g + GSS_CLS_L2PF pulled into L2 (one 128-byte line per lane): the register
+    // prefetch above then waits for L2 rather than DRAM, without holding more registers
+    if (g + GSS_CLS_L2PF < nfull && lane * 128u < U * 32u * (uint32_t)sizeof(Key))
+      asm volatile("prefetch.global.L2 [%0];" ::"l"(reinterpret_cast<const char*>(sp - lane) +
+                                                  ((size_t)(g + GSS_CLS_L2PF) * G) * sizeof(Key) + lane * 128u));
+#endif
     uint32_t id[U];
     ids_of(e, id);
 #pragma unroll
@@ -1443,9 +1453,9 @@ __device__ __forceinline__ void bulk_g2s(uint32_t sdst, const void* gsrc, uint32
 #ifndef GSS_SCATTER_IO_WARPS
 #define GSS_SCATTER_IO_WARPS 2   // one I/O warp could not keep up with the stores (rank warps waited on it)
 #endif
-template <class Key, class IdT>
+template <class Key, class IdT, int NIO_ = GSS_SCATTER_IO_WARPS>
 struct ScatterWsSmem {
-  static constexpr uint32_t NIO = GSS_SCATTER_IO_WARPS;                    // I/O warps
+  static constexpr uint32_t NIO = NIO_;                                    // I/O warps
   static constexpr uint32_t NR = kScatterThreads / 32 - NIO;               // rank warps
   static constexpr uint32_t ITER = GSS_SCATTER_ITER;
   static constexpr uint32_t C = NR * 32 * ITER;                            // keys per chunk
@@ -1460,11 +1470,11 @@ struct ScatterWsSmem {
   __host__ __device__ static size_t bytes(uint32_t kmax) { return 2 * in_bytes() + stage_bytes() + head_bytes(kmax); }
 };
 
-template <class Key, class Val, class IdT>
+template <class Key, class Val, class IdT, int NIO = GSS_SCATTER_IO_WARPS>
 __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   static_assert(!kHasVal<Val>, "keys only");
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  using SM = ScatterWsSmem<Key, IdT>;
+  using SM = ScatterWsSmem<Key, IdT, NIO>;
   constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, NRT = NR * 32, NIOT = SM::NIO * 32;
   // named barriers: 1 the rank warps; 2 staged (rank warps arrive, I/O syncs); 3 staging free (I/O arrives,
   // rank warps sync); 4+b input buffer b read (rank warps arrive, I/O syncs)
