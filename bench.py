@@ -278,6 +278,36 @@ def run_reference(args, wl):
 # ---------------------------------------------------------------------------
 # our arm
 # ---------------------------------------------------------------------------
+def library_ref(torch, dkeys, dvals, bits, pairs, steps, dev, stream) -> dict:
+    """torch.sort (CUB's device radix sort) of the same device keys -- context for the sample sort, not part of
+    it: unsigned keys sorted through the order-preserving signed view (top bit flipped outside the timing);
+    pairs as sort + gather of the values by the returned permutation."""
+    try:
+        sd = torch.int64 if bits == 64 else torch.int32
+        flip = torch.tensor(-(1 << (bits - 1)), dtype=sd, device=dev)
+        ks = dkeys.view(sd) ^ flip
+        def once():
+            y, idx = torch.sort(ks)
+            if pairs:
+                dvals.view(sd).index_select(0, idx)
+            return y
+        for _ in range(2):
+            y = once()
+        torch.cuda.synchronize(dev)
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        k = max(3, min(steps, 10))
+        e0.record(stream)
+        for _ in range(k):
+            once()
+        e1.record(stream)
+        torch.cuda.synchronize(dev)
+        ms = e0.elapsed_time(e1) / k
+        return {"what": "torch.sort (CUB device radix sort) of the same resident keys" + (" + value gather" if pairs else ""),
+                "ms_per_step": round(ms, 4), "value": round(dkeys.numel() / (ms * 1e-3) / 1e9, 3), "unit": "Gkeys/s"}
+    except Exception as e:  # pragma: no cover - context only
+        return {"error": str(e)[:200]}
+
+
 def run_single(args, wl):
     os.environ.setdefault("NCCL_DEBUG", "WARN")          # keep stdout to the one JSON line
     import torch
@@ -369,6 +399,9 @@ def run_single(args, wl):
                                         "frac": round(B / (hbm * 1e9) / (ms * 1e-3), 4),
                                         "levels": st.levels, "split_elems": st.split_elems[: max(st.levels, 1)],
                                         "small_buckets": st.small_buckets}
+    # ---- GPU library context: torch.sort (CUB device radix sort) on the same resident keys ----
+    if not use_dist and not args.no_library_ref:
+        extra["gpu_library_ref"] = library_ref(torch, dkeys, dvals, bits, pairs, args.steps, dev, stream)
     # ---- end to end through the C ABI with host buffers ----
     e2e = None
     if not use_dist:
@@ -588,6 +621,7 @@ def main():
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--workload", default=DEFAULT_WORKLOAD, choices=sorted(WORKLOADS))
     ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-library-ref", action="store_true", help="skip the torch.sort (CUB) context timing")
     ap.add_argument("--force-dist", action="store_true", help="use the distributed path even on one GPU")
     ap.add_argument("--fused", action="store_true", help="distributed path: fused scatter into peer windows "
                                                          "(GSS_FLAG_DIST_FUSED)")
