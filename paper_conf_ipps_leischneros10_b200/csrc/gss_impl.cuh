@@ -402,18 +402,23 @@ struct Engine {
     auto kws = k_scatter_bulk<Key, Val, IdT, 1>;
     size_t sm_ws = 0;
     int g_ws = 0;
-    if constexpr (!kHasVal<Val>) {
-      // 14 rank + 2 I/O warps; where their chunk buffers do not fit two CTAs per SM (k = 512, 16-bit ids),
-      // 12 + 4 (shorter chunks)
+    {
+      // keys alone and 8-byte pairs: 14 rank + 2 I/O warps; where their chunk buffers do not fit two CTAs per SM
+      // (k = 512 with 16-bit ids; 4-byte keys, 16 per lane), 12 + 4 (shorter chunks).  16-byte pairs keep the
+      // single-role scatter: with values their chunks shrink to 4 keys per lane, and that measured slower
+      // (2^27 u64 pairs 3.64 vs 3.01 ms; u32 keys 0.83 vs 1.06, u32 pairs 1.94 vs 2.01, profiles/r02_ab_scatter_ws_kinds.log)
       constexpr size_t kWsMax = 113 * 1024;
-      const bool ok = use_bulk && !c.nremote && kmax <= 512 && !(cfg.flags & (kFlagScatterCtaCounters | kFlagScatterNoWs));
-      if (ok && ScatterWsSmem<Key, IdT>::bytes(kmax) <= kWsMax) {
+      constexpr bool kWsKind = !kHasVal<Val> || sizeof(Key) + sizeof(Val) <= 8;
+      const bool ok = kWsKind && !c.nremote && !c.stable && !c.recompute && kmax <= 512 &&
+                      !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS | kFlagScatterCtaCounters |
+                                     kFlagScatterNoWs));
+      if (ok && ScatterWsSmem<Key, Val, IdT>::bytes(kmax) <= kWsMax) {
         use_ws = true;
-        sm_ws = ScatterWsSmem<Key, IdT>::bytes(kmax);
+        sm_ws = ScatterWsSmem<Key, Val, IdT>::bytes(kmax);
         kws = k_scatter_ws<Key, Val, IdT>;
-      } else if (ok && ScatterWsSmem<Key, IdT, 4>::bytes(kmax) <= kWsMax) {
+      } else if (ok && ScatterWsSmem<Key, Val, IdT, 4>::bytes(kmax) <= kWsMax) {
         use_ws = true;
-        sm_ws = ScatterWsSmem<Key, IdT, 4>::bytes(kmax);
+        sm_ws = ScatterWsSmem<Key, Val, IdT, 4>::bytes(kmax);
         kws = k_scatter_ws<Key, Val, IdT, 4>;
       }
       if (use_ws) {

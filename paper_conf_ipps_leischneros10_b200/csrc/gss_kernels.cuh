@@ -1453,16 +1453,28 @@ __device__ __forceinline__ void bulk_g2s(uint32_t sdst, const void* gsrc, uint32
 #ifndef GSS_SCATTER_IO_WARPS
 #define GSS_SCATTER_IO_WARPS 2   // one I/O warp could not keep up with the stores (rank warps waited on it)
 #endif
-template <class Key, class IdT, int NIO_ = GSS_SCATTER_IO_WARPS>
+#ifndef GSS_SCATTER_ITER_WS_KV
+#define GSS_SCATTER_ITER_WS_KV 4   // 16-byte pairs: keys per lane (the values double the chunk buffers)
+#endif
+template <class Key, class Val, class IdT, int NIO_ = GSS_SCATTER_IO_WARPS>
 struct ScatterWsSmem {
   static constexpr uint32_t NIO = NIO_;                                    // I/O warps
   static constexpr uint32_t NR = kScatterThreads / 32 - NIO;               // rank warps
-  static constexpr uint32_t ITER = GSS_SCATTER_ITER;
+  static constexpr bool KV = kHasVal<Val>;
+  static constexpr uint32_t ITER =                                         // keys per lane
+      KV ? (sizeof(Key) + sizeof(Val) <= 8 ? GSS_SCATTER_ITER : GSS_SCATTER_ITER_WS_KV)
+         : (sizeof(Key) == 4 ? GSS_SCATTER_ITER_U32 : GSS_SCATTER_ITER);
   static constexpr uint32_t C = NR * 32 * ITER;                            // keys per chunk
   static constexpr uint32_t A = 16 / sizeof(Key);
+  static constexpr uint32_t VS = KV ? (uint32_t)sizeof(Val) : 0u;          // value bytes
+  static constexpr uint32_t AV = KV ? 16u / VS : 1u;
   static constexpr size_t al(size_t x) { return (x + 15) & ~size_t(15); }
-  static constexpr size_t in_bytes() { return al((size_t)(C + A) * sizeof(Key)) + al((size_t)C * sizeof(IdT)); }
-  static constexpr size_t stage_bytes() { return al((size_t)C * sizeof(Key)) + al((size_t)C * sizeof(IdT)); }
+  static constexpr size_t ink_bytes() { return al((size_t)(C + A) * sizeof(Key)); }
+  static constexpr size_t inv_bytes() { return KV ? al((size_t)(C + AV) * VS) : 0; }
+  static constexpr size_t in_bytes() { return ink_bytes() + inv_bytes() + al((size_t)C * sizeof(IdT)); }
+  static constexpr size_t stage_bytes() {
+    return al((size_t)C * sizeof(Key)) + (KV ? al((size_t)C * VS) : 0) + al((size_t)C * sizeof(IdT));
+  }
   // counters NR x kmax/2 words; gbase kmax; delta 2 x kmax; scan 64 words; 2 mbarriers
   __host__ __device__ static size_t head_bytes(uint32_t kmax) {
     return al(((size_t)NR * ((kmax + 1) / 2) + 3 * (size_t)kmax + 64) * 4 + 32);
@@ -1472,20 +1484,24 @@ struct ScatterWsSmem {
 
 template <class Key, class Val, class IdT, int NIO = GSS_SCATTER_IO_WARPS>
 __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
-  static_assert(!kHasVal<Val>, "keys only");
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  using SM = ScatterWsSmem<Key, IdT, NIO>;
-  constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, NRT = NR * 32, NIOT = SM::NIO * 32;
+  using SM = ScatterWsSmem<Key, Val, IdT, NIO>;
+  constexpr bool KV = SM::KV;
+  constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, AV = SM::AV, NRT = NR * 32,
+                     NIOT = SM::NIO * 32;
   // named barriers: 1 the rank warps; 2 staged (rank warps arrive, I/O syncs); 3 staging free (I/O arrives,
   // rank warps sync); 4+b input buffer b read (rank warps arrive, I/O syncs)
   constexpr uint32_t BAR_RANK = 1, BAR_STAGED = 2, BAR_FREE = 3, BAR_IN = 4;
   // input buffer b (selected arithmetically: no local-memory arrays)
   auto ink = [&](uint32_t b) { return reinterpret_cast<Key*>(smem_raw + b * SM::in_bytes()); };
+  auto inv = [&](uint32_t b) { return reinterpret_cast<Val*>(smem_raw + b * SM::in_bytes() + SM::ink_bytes()); };
   auto ini = [&](uint32_t b) {
-    return reinterpret_cast<IdT*>(smem_raw + b * SM::in_bytes() + SM::al((size_t)(C + A) * sizeof(Key)));
+    return reinterpret_cast<IdT*>(smem_raw + b * SM::in_bytes() + SM::ink_bytes() + SM::inv_bytes());
   };
   Key* stk = reinterpret_cast<Key*>(smem_raw + 2 * SM::in_bytes());
-  IdT* sti = reinterpret_cast<IdT*>(smem_raw + 2 * SM::in_bytes() + SM::al((size_t)C * sizeof(Key)));
+  Val* stv = reinterpret_cast<Val*>(smem_raw + 2 * SM::in_bytes() + SM::al((size_t)C * sizeof(Key)));
+  IdT* sti = reinterpret_cast<IdT*>(smem_raw + 2 * SM::in_bytes() + SM::al((size_t)C * sizeof(Key)) +
+                                    (KV ? SM::al((size_t)C * SM::VS) : 0));
   const uint32_t KH = (kmax + 1) / 2;
   uint32_t* cnt = reinterpret_cast<uint32_t*>(smem_raw + 2 * SM::in_bytes() + SM::stage_bytes());
   uint32_t* gbase = cnt + NR * KH;                       // next global index of each id (owner threads)
@@ -1498,6 +1514,9 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
   const uint32_t nt = c.cnt->lvl[level].num_tiles;
   const Key* ksrc = c.keys(c.src(level));
   Key* kdst = c.wkeys(c.dst(level));
+  const Val* vsrc = nullptr;
+  Val* vdst = nullptr;
+  if constexpr (KV) { vsrc = c.vals(c.src(level)); vdst = c.wvals(c.dst(level)); }
   const IdT* idsrc = c.ids;
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   if (blockIdx.x >= nt) return;
@@ -1551,10 +1570,24 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
       for (uint32_t q = lane; q < h; q += 32) bk[q + sh] = ksrc[g0 + q];
       for (uint32_t q = h + mid + lane; q < clen; q += 32) bk[q + sh] = ksrc[g0 + q];
       for (uint32_t q = ib / (uint32_t)sizeof(IdT) + lane; q < clen; q += 32) bi[q] = idsrc[u.idb + u.c0 + q];
+      uint32_t shv = 0, hv = 0, midv = 0;
+      if constexpr (KV) {                                // values: their own 16-byte phase
+        shv = g0 & (AV - 1);
+        hv = min(clen, (AV - shv) & (AV - 1));
+        midv = (clen - hv) & ~(AV - 1);
+        Val* bv = inv(b);
+        for (uint32_t q = lane; q < hv; q += 32) bv[q + shv] = vsrc[g0 + q];
+        for (uint32_t q = hv + midv + lane; q < clen; q += 32) bv[q + shv] = vsrc[g0 + q];
+      }
       __syncwarp();
       if (lane == 0) {
         fence_proxy_async_smem();                        // the buffer's generic accesses before the async writes
-        wsync::mbar_arrive_tx(mbar(b), mid * (uint32_t)sizeof(Key) + ib);
+        wsync::mbar_arrive_tx(mbar(b), mid * (uint32_t)sizeof(Key) + ib + midv * SM::VS);
+        if constexpr (KV) {
+          if (midv)
+            wsync::bulk_g2s((uint32_t)__cvta_generic_to_shared(inv(b) + hv + shv), vsrc + g0 + hv, midv * SM::VS,
+                            mbar(b));
+        }
         if (mid)
           wsync::bulk_g2s((uint32_t)__cvta_generic_to_shared(bk + h + sh), ksrc + g0 + h, mid * (uint32_t)sizeof(Key),
                           mbar(b));
@@ -1582,8 +1615,16 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         for (int u = 0; u < 4; u++) { x[u] = stk[s + NIOT * u]; y[u] = s + NIOT * u + dl[sti[s + NIOT * u]]; }
 #pragma unroll
         for (int u = 0; u < 4; u++) kdst[y[u]] = x[u];
+        if constexpr (KV) {
+#pragma unroll
+          for (int u = 0; u < 4; u++) vdst[y[u]] = stv[s + NIOT * u];
+        }
       }
-      for (; s < clen; s += NIOT) kdst[s + dl[sti[s]]] = stk[s];
+      for (; s < clen; s += NIOT) {
+        const uint32_t y = s + dl[sti[s]];
+        kdst[y] = stk[s];
+        if constexpr (KV) vdst[y] = stv[s];
+      }
       __syncwarp();
       wsync::bar_arrive(BAR_FREE, kScatterThreads);      // the staging buffer may be rewritten
       advance(cur);
@@ -1611,10 +1652,11 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
       }
     }
     const uint32_t clen = min(C, cur.len - cur.c0);
-    const uint32_t sh = (cur.beg + cur.c0) & (A - 1);
+    const uint32_t sh = (cur.beg + cur.c0) & (A - 1), shv = (cur.beg + cur.c0) & (AV - 1);
     for (uint32_t j = lane; j < KP; j += 32) cnt[w * KH + j] = 0;
     wsync::mbar_wait(mbar(b), (k >> 1) & 1);
     Key kk[ITER];
+    Val vv[ITER];
     uint32_t iid[ITER];
     {
       const Key* bk = ink(b);
@@ -1625,6 +1667,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         iid[it] = 0xffffffffu;
         if (q < clen) {
           kk[it] = bk[q + sh];
+          if constexpr (KV) vv[it] = inv(b)[q + shv];
           iid[it] = bi[q];
         }
       }
@@ -1714,6 +1757,7 @@ __global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val,
         const uint32_t id = iid[it] & 0xffffu;
         const uint32_t pos = ((wc[id >> 1] >> (16 * (id & 1))) & 0xffffu) + (iid[it] >> 16);
         stk[pos] = kk[it];
+        if constexpr (KV) stv[pos] = vv[it];
         sti[pos] = (IdT)id;
       }
     }
