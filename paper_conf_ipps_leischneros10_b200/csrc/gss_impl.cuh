@@ -403,16 +403,24 @@ struct Engine {
     size_t sm_ws = 0;
     int g_ws = 0;
     {
-      // keys alone and 8-byte pairs: 14 rank + 2 I/O warps; where their chunk buffers do not fit two CTAs per SM
-      // (k = 512 with 16-bit ids; 4-byte keys, 16 per lane), 12 + 4 (shorter chunks).  16-byte pairs keep the
-      // single-role scatter: with values their chunks shrink to 4 keys per lane, and that measured slower
-      // (2^27 u64 pairs 3.64 vs 3.01 ms; u32 keys 0.83 vs 1.06, u32 pairs 1.94 vs 2.01, profiles/r02_ab_scatter_ws_kinds.log)
+      // keys alone and 8-byte pairs: 14 rank + 2 I/O warps, two CTAs per SM; where their chunk buffers do not
+      // fit (k = 512 with 16-bit ids; 4-byte keys, 16 per lane), 12 + 4 (shorter chunks).  16-byte pairs: two
+      // CTAs per SM would leave 4 keys per lane, which measured slower than the single-role kernel (2^27 u64
+      // pairs 3.64 vs 3.01 ms; u32 keys 0.83 vs 1.06, u32 pairs 1.94 vs 2.01,
+      // profiles/r02_ab_scatter_ws_kinds.log), so they run one CTA per SM (profiles/r02_ab_scatter_ws_pairs.log)
       constexpr size_t kWsMax = 113 * 1024;
       constexpr bool kWsKind = !kHasVal<Val> || sizeof(Key) + sizeof(Val) <= 8;
-      const bool ok = kWsKind && !c.nremote && !c.stable && !c.recompute && kmax <= 512 &&
-                      !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS | kFlagScatterCtaCounters |
-                                     kFlagScatterNoWs));
-      if (ok && ScatterWsSmem<Key, Val, IdT>::bytes(kmax) <= kWsMax) {
+      const bool ok0 = !c.nremote && !c.stable && !c.recompute && kmax <= 512 &&
+                       !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS | kFlagScatterCtaCounters |
+                                      kFlagScatterNoWs));
+      const bool ok = kWsKind && ok0;
+      if (!kWsKind && ok0 && ScatterWsSmem<Key, Val, IdT, GSS_SCATTER_IO_WARPS, true>::bytes(kmax) <= 227 * 1024) {
+        // 16-byte pairs: one CTA per SM with the whole shared memory and 8 keys per lane (2^27 u64 pairs:
+        // scatter 3.02 -> 2.57 ms, 2^29 at k = 512 16.7 -> 15.1; with two CTAs and 4 keys per lane it lost)
+        use_ws = true;
+        sm_ws = ScatterWsSmem<Key, Val, IdT, GSS_SCATTER_IO_WARPS, true>::bytes(kmax);
+        kws = k_scatter_ws<Key, Val, IdT, GSS_SCATTER_IO_WARPS, true>;
+      } else if (ok && ScatterWsSmem<Key, Val, IdT>::bytes(kmax) <= kWsMax) {
         use_ws = true;
         sm_ws = ScatterWsSmem<Key, Val, IdT>::bytes(kmax);
         kws = k_scatter_ws<Key, Val, IdT>;

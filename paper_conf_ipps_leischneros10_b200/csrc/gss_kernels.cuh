@@ -1456,13 +1456,14 @@ __device__ __forceinline__ void bulk_g2s(uint32_t sdst, const void* gsrc, uint32
 #ifndef GSS_SCATTER_ITER_WS_KV
 #define GSS_SCATTER_ITER_WS_KV 4   // 16-byte pairs: keys per lane (the values double the chunk buffers)
 #endif
-template <class Key, class Val, class IdT, int NIO_ = GSS_SCATTER_IO_WARPS>
+template <class Key, class Val, class IdT, int NIO_ = GSS_SCATTER_IO_WARPS, bool ONE_ = false>
 struct ScatterWsSmem {
   static constexpr uint32_t NIO = NIO_;                                    // I/O warps
   static constexpr uint32_t NR = kScatterThreads / 32 - NIO;               // rank warps
   static constexpr bool KV = kHasVal<Val>;
+  // ONE_: one CTA per SM with the whole shared memory (16-byte pairs at 8 keys per lane)
   static constexpr uint32_t ITER =                                         // keys per lane
-      KV ? (sizeof(Key) + sizeof(Val) <= 8 ? GSS_SCATTER_ITER : GSS_SCATTER_ITER_WS_KV)
+      KV ? (sizeof(Key) + sizeof(Val) <= 8 || ONE_ ? GSS_SCATTER_ITER : GSS_SCATTER_ITER_WS_KV)
          : (sizeof(Key) == 4 ? GSS_SCATTER_ITER_U32 : GSS_SCATTER_ITER);
   static constexpr uint32_t C = NR * 32 * ITER;                            // keys per chunk
   static constexpr uint32_t A = 16 / sizeof(Key);
@@ -1482,10 +1483,11 @@ struct ScatterWsSmem {
   __host__ __device__ static size_t bytes(uint32_t kmax) { return 2 * in_bytes() + stage_bytes() + head_bytes(kmax); }
 };
 
-template <class Key, class Val, class IdT, int NIO = GSS_SCATTER_IO_WARPS>
-__global__ void __launch_bounds__(kScatterThreads, 2) k_scatter_ws(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
+template <class Key, class Val, class IdT, int NIO = GSS_SCATTER_IO_WARPS, bool ONE = false>
+__global__ void __launch_bounds__(kScatterThreads, ONE ? 1 : 2)
+    k_scatter_ws(Ctx<Key, Val, IdT> c, uint32_t level, uint32_t kmax) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  using SM = ScatterWsSmem<Key, Val, IdT, NIO>;
+  using SM = ScatterWsSmem<Key, Val, IdT, NIO, ONE>;
   constexpr bool KV = SM::KV;
   constexpr uint32_t NR = SM::NR, ITER = SM::ITER, C = SM::C, A = SM::A, AV = SM::AV, NRT = NR * 32,
                      NIOT = SM::NIO * 32;
