@@ -37,6 +37,7 @@ namespace gssh {
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
 inline constexpr uint32_t kFlagScatterBulk = 1u << 29;          // ablation: bulk-copy scatter for 4-byte keys too
+inline constexpr uint32_t kFlagScatterWsOne = 1u << 26;         // ablation: keys alone through the one-CTA/SM form too
 inline constexpr uint32_t kFlagScatterNoWs = 1u << 27;          // ablation: the single-role bulk scatter (k_scatter_bulk)
 inline constexpr uint32_t kFlagSmallNarrow = 1u << 28;          // ablation: 48-register block sort for classes <= 20 warps
                                                                 // (2^28 u64: 4.98 vs 4.90 ms -- occupancy is not the limit)
@@ -414,7 +415,8 @@ struct Engine {
                        !(cfg.flags & (GSS_FLAG_DIRECT_SCATTER | GSS_FLAG_SCATTER_REGS | kFlagScatterCtaCounters |
                                       kFlagScatterNoWs));
       const bool ok = kWsKind && ok0;
-      if (!kWsKind && ok0 && ScatterWsSmem<Key, Val, IdT, GSS_SCATTER_IO_WARPS, true>::bytes(kmax) <= 227 * 1024) {
+      if ((!kWsKind || (cfg.flags & kFlagScatterWsOne)) && ok0 &&
+          ScatterWsSmem<Key, Val, IdT, GSS_SCATTER_IO_WARPS, true>::bytes(kmax) <= 227 * 1024) {
         // 16-byte pairs: one CTA per SM with the whole shared memory and 8 keys per lane (2^27 u64 pairs:
         // scatter 3.02 -> 2.57 ms, 2^29 at k = 512 16.7 -> 15.1; with two CTAs and 4 keys per lane it lost)
         use_ws = true;

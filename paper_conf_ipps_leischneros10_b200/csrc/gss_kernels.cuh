@@ -480,7 +480,10 @@ __device__ __forceinline__ void classify_tile(const Key* __restrict__ src, IdT* 
                                               uint32_t ks, uint32_t K, uint32_t wc_s, IdT* wid, Cmp less) {
   auto ids_of = [&](const Key (&e)[GSS_CLS_U], uint32_t (&id)[GSS_CLS_U]) {
     if constexpr (LUT) {
-      if (cs.use_lut) lut_group<MODE>(e, id, cs.lut_s, spl, cs.base, cs.shift, ks);
+#ifndef GSS_CLS_LUT_ONLY
+#define GSS_CLS_LUT_ONLY 0   // experiment: no per-bucket fallback to the descent in the lookup instantiation
+#endif
+      if (GSS_CLS_LUT_ONLY || cs.use_lut) lut_group<MODE>(e, id, cs.lut_s, spl, cs.base, cs.shift, ks);
       else descend_group<MODE>(e, id, cs.tree_s, cs.rep_b, spl, cs.logk, ks, K, less);
     } else {
       descend_group<MODE>(e, id, cs.tree_s, cs.rep_b, spl, cs.logk, ks, K, less);
@@ -1464,7 +1467,7 @@ struct ScatterWsSmem {
   // ONE_: one CTA per SM with the whole shared memory (16-byte pairs at 8 keys per lane)
   static constexpr uint32_t ITER =                                         // keys per lane
       KV ? (sizeof(Key) + sizeof(Val) <= 8 || ONE_ ? GSS_SCATTER_ITER : GSS_SCATTER_ITER_WS_KV)
-         : (sizeof(Key) == 4 ? GSS_SCATTER_ITER_U32 : GSS_SCATTER_ITER);
+         : (sizeof(Key) == 4 ? GSS_SCATTER_ITER_U32 : GSS_SCATTER_ITER) * (ONE_ ? 2 : 1);
   static constexpr uint32_t C = NR * 32 * ITER;                            // keys per chunk
   static constexpr uint32_t A = 16 / sizeof(Key);
   static constexpr uint32_t VS = KV ? (uint32_t)sizeof(Val) : 0u;          // value bytes
