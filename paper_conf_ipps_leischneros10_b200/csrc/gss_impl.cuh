@@ -37,6 +37,7 @@ namespace gssh {
 inline constexpr uint32_t kVersion = 1;
 inline constexpr uint32_t kFlagScatterCtaCounters = 1u << 30;   // ablation: ranks from one counter set per CTA (k_scatter_fast)
 inline constexpr uint32_t kFlagScatterBulk = 1u << 29;          // ablation: bulk-copy scatter for 4-byte keys too
+inline constexpr uint32_t kFlagSampleFull = 1u << 25;          // ablation: 1024-thread sample sorts always
 inline constexpr uint32_t kFlagScatterWsOne = 1u << 26;         // ablation: keys alone through the one-CTA/SM form too
 inline constexpr uint32_t kFlagScatterNoWs = 1u << 27;          // ablation: the single-role bulk scatter (k_scatter_bulk)
 inline constexpr uint32_t kFlagSmallNarrow = 1u << 28;          // ablation: 48-register block sort for classes <= 20 warps
@@ -355,8 +356,12 @@ struct Engine {
       GSS_TRY(launch(prof, GSS_K_INIT, s, count, [&] { k_init<Key, Val, IdT><<<1, 256, 0, s>>>(c); }));
     const uint32_t kmax = cfg.kmax;
     // kernels and their shared-memory sizes
-    auto ks = k_sample<Key, Val, IdT, Cmp>;
-    const size_t sm_sample = CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
+    // the sample sort CTA: 512 threads (two per SM) when every bucket's a * k_b sample fits 8192 keys
+    const bool half_sample = (uint64_t)cfg.a * kmax <= 8192 && !(cfg.flags & kFlagSampleFull);
+    auto ks = half_sample ? k_sample<Key, Val, IdT, Cmp, kSampleThreads / 2> : k_sample<Key, Val, IdT, Cmp>;
+    const int nt_sample = half_sample ? kSampleThreads / 2 : kSampleThreads;
+    const size_t sm_sample = half_sample ? CtaSort<Key, NoVal, kSampleThreads / 2, Cmp>::smem_bytes()
+                                         : CtaSort<Key, NoVal, kSampleThreads, Cmp>::smem_bytes();
     auto kc = mode == MODE_PARTITION_BY ? k_classify<Key, Val, IdT, Cmp, true> : k_classify<Key, Val, IdT, Cmp, false>;
     if constexpr (lut_ok<Key, Cmp>()) {
       if (mode != MODE_PARTITION_BY && c.lut) kc = k_classify<Key, Val, IdT, Cmp, false, true>;   // radix-indexed lookup
@@ -368,9 +373,9 @@ struct Engine {
     GSS_TRY(set_smem(ks, sm_sample));
     GSS_TRY(set_smem(kc, sm_cls));
     GSS_TRY(set_smem(ksc, sm_sc));
-    static GridCache gc_sample, gc_plan;
-    int g_sample = gc_sample.get(di.dev), g_plan = gc_plan.get(di.dev);
-    if (!g_sample) { g_sample = grid_for(ks, kSampleThreads, sm_sample, di.sms); gc_sample.put(di.dev, g_sample); }
+    static GridCache gc_sample[2], gc_plan;
+    int g_sample = gc_sample[half_sample].get(di.dev), g_plan = gc_plan.get(di.dev);
+    if (!g_sample) { g_sample = grid_for(ks, nt_sample, sm_sample, di.sms); gc_sample[half_sample].put(di.dev, g_sample); }
     if (!g_plan) { g_plan = grid_for(k_plan<Key, Val, IdT>, kPlanThreads, 0, di.sms); gc_plan.put(di.dev, g_plan); }
     const int g_cls = grid_for(kc, kClsThreads, sm_cls, di.sms);
     const int g_sc = grid_for(ksc, kScatterThreads, sm_sc, di.sms);
@@ -445,7 +450,7 @@ struct Engine {
       if (mode == MODE_PARTITION_BY) {
         GSS_TRY(launch(prof, GSS_K_SAMPLE, s, count, [&] { k_set_splitters<Key, Val, IdT><<<1, 256, 0, s>>>(c); }));
       } else {
-        GSS_TRY(launch(prof, GSS_K_SAMPLE, s, count, [&] { ks<<<g_sample, kSampleThreads, sm_sample, s>>>(c, l); }));
+        GSS_TRY(launch(prof, GSS_K_SAMPLE, s, count, [&] { ks<<<g_sample, nt_sample, sm_sample, s>>>(c, l); }));
       }
       GSS_TRY(launch(prof, GSS_K_CLASSIFY, s, count, [&] { kc<<<g_cls, kClsThreads, sm_cls, s>>>(c, l, kmax); }));
       GSS_TRY(launch(prof, GSS_K_SCAN, s, count,

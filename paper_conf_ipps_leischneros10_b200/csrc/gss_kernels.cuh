@@ -111,11 +111,14 @@ __global__ void k_init(Ctx<Key, Val, IdT> c) {
 // (R4), then k_s = k_b/2 splitters S[(s/k_s)(i+1)-1]; the implicit tree
 // bt[j] = s_{(2q+1) k_s / 2^(d+1)}.
 // ---------------------------------------------------------------------------
-template <class Key, class Val, class IdT, class Cmp>
-__global__ void __launch_bounds__(kSampleThreads, 1) k_sample(Ctx<Key, Val, IdT> c, uint32_t level) {
+// NT: 1024 threads (capacity 16384 sample keys), or 512 (8192) with two CTAs per SM where a * k_max fits,
+// so that the 256 sample sorts of a level with k = 256 run in one wave
+template <class Key, class Val, class IdT, class Cmp, int NT = kSampleThreads>
+__global__ void __launch_bounds__(NT, kSampleThreads / NT) k_sample(Ctx<Key, Val, IdT> c, uint32_t level) {
+  constexpr int kSampleThreads = NT;
   extern __shared__ __align__(16) unsigned char smem_raw[];
   Key* sk = reinterpret_cast<Key*>(smem_raw);
-  using Sorter = CtaSort<Key, NoVal, kSampleThreads, Cmp>;
+  using Sorter = CtaSort<Key, NoVal, NT, Cmp>;
   const Cmp less;
   const uint32_t slot = level & 1;
   const uint32_t nb = c.cnt->lvl[level].num_buckets;
