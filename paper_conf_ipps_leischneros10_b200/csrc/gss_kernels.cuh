@@ -1459,6 +1459,9 @@ __device__ __forceinline__ void bulk_g2s(uint32_t sdst, const void* gsrc, uint32
 #ifndef GSS_SCATTER_IO_WARPS
 #define GSS_SCATTER_IO_WARPS 2   // one I/O warp could not keep up with the stores (rank warps waited on it)
 #endif
+#ifndef GSS_WS_FOLD2
+#define GSS_WS_FOLD2 0   // 1: two threads per id pair in the fold (measured slower: u32 0.88 vs 0.83 ms, sorted u64 1.84 vs 1.63)
+#endif
 #ifndef GSS_SCATTER_ITER_WS_KV
 #define GSS_SCATTER_ITER_WS_KV 4   // 16-byte pairs: keys per lane (the values double the chunk buffers)
 #endif
@@ -1648,14 +1651,19 @@ __global__ void __launch_bounds__(kScatterThreads, ONE ? 1 : 2)
   for (uint32_t k = 0;; k++) {
     const uint32_t b = k & 1;
     const uint32_t K = cur.K, KP = (K + 1) / 2;
-    if (cur.c0 == 0 && own < KP) {                       // a new tile: the global start of each id in it
+    // owner of id pair (2pp, 2pp+1): thread pp, or threads 2pp (hh = 0) and 2pp+1 (hh = 1) where 2 KP
+    // threads exist (the fold below); gbase of a pair is read and written by its hh = 0 thread only
+    const bool two = GSS_WS_FOLD2 && 2 * KP <= NRT;      // block-uniform
+    const uint32_t pp = two ? own >> 1 : own, hh = two ? (own & 1) : 0u;
+    const bool act = pp < KP;
+    if (cur.c0 == 0 && act && hh == 0) {                 // a new tile: the global start of each id in it
       const Bucket B = c.bk[slot][c.tile_bucket[slot][cur.t]];
       const uint32_t tl = cur.t - B.tile_start;
       const uint32_t* hist = c.hist[slot] + B.hist_base;
       const uint32_t hb = hist[0];
 #pragma unroll
       for (uint32_t j = 0; j < 2; j++) {
-        const uint32_t id = 2 * own + j;
+        const uint32_t id = 2 * pp + j;
         if (id < K) gbase[id] = hist[id * B.ntiles + tl] - hb + B.lo;
       }
     }
@@ -1704,17 +1712,26 @@ __global__ void __launch_bounds__(kScatterThreads, ONE ? 1 : 2)
       }
     }
     wsync::bar_sync(BAR_RANK, NRT);                      // counters complete
-    // owners: chunk totals of ids 2*own, 2*own+1 (runs packed in id order), every warp's start in them
-    uint32_t L0 = 0, L1 = 0;
-    if (own < KP) {
-#pragma unroll
-      for (uint32_t q = 0; q < NR; q++) {
-        const uint32_t x = cnt[q * KH + own];
-        L0 += x & 0xffffu;
-        L1 += x >> 16;
+    // owners: chunk totals of ids 2p, 2p+1 (runs packed in id order), every warp's start in them.  Two
+    // adjacent threads per pair (each folding half of the rank warps' counters) where 2 * KP threads exist,
+    // which halves the serial fold between the barriers; else one thread per pair.
+    const uint32_t qa = two ? hh * (NR / 2) : 0u, qb = two ? (hh ? NR : NR / 2) : NR;
+    uint32_t a0 = 0, a1 = 0;                              // this thread's warps
+    if (act) {
+#pragma unroll 7
+      for (uint32_t q = qa; q < qb; q++) {
+        const uint32_t x = cnt[q * KH + pp];
+        a0 += x & 0xffffu;
+        a1 += x >> 16;
       }
     }
-    const uint32_t tsum = L0 + L1;                       // an odd K's missing id counts 0
+    uint32_t b0 = 0, b1 = 0;                              // the partner's warps
+    if (two) {
+      b0 = __shfl_xor_sync(kFull, a0, 1);
+      b1 = __shfl_xor_sync(kFull, a1, 1);
+    }
+    const uint32_t L0 = a0 + b0, L1 = a1 + b1;
+    const uint32_t tsum = (act && hh == 0) ? L0 + L1 : 0u;   // an odd K's missing id counts 0
     uint32_t ex;
     {
       uint32_t inc = tsum;
@@ -1738,21 +1755,24 @@ __global__ void __launch_bounds__(kScatterThreads, ONE ? 1 : 2)
       wsync::bar_sync(BAR_RANK, NRT);
       ex = s_warp[32 + w] + inc - tsum;
     }
-    if (own < KP) {
-      uint32_t* dl = delta + b * kmax;
+    if (two) ex = __shfl_sync(kFull, ex, lane & ~1);     // the pair's base (its even thread's prefix)
+    if (act) {
       const uint32_t st0 = ex, st1 = ex + L0;
-      const uint32_t id0 = 2 * own;
-      dl[id0] = gbase[id0] - st0;
-      gbase[id0] += L0;
-      if (id0 + 1 < K) {
-        dl[id0 + 1] = gbase[id0 + 1] - st1;
-        gbase[id0 + 1] += L1;
+      const uint32_t id0 = 2 * pp;
+      if (hh == 0) {
+        uint32_t* dl = delta + b * kmax;
+        dl[id0] = gbase[id0] - st0;
+        gbase[id0] += L0;
+        if (id0 + 1 < K) {
+          dl[id0 + 1] = gbase[id0 + 1] - st1;
+          gbase[id0 + 1] += L1;
+        }
       }
-      uint32_t r0 = st0, r1 = st1;
-#pragma unroll
-      for (uint32_t q = 0; q < NR; q++) {
-        const uint32_t x = cnt[q * KH + own];
-        cnt[q * KH + own] = r0 | (r1 << 16);
+      uint32_t r0 = st0 + (hh ? b0 : 0u), r1 = st1 + (hh ? b1 : 0u);
+#pragma unroll 7
+      for (uint32_t q = qa; q < qb; q++) {
+        const uint32_t x = cnt[q * KH + pp];
+        cnt[q * KH + pp] = r0 | (r1 << 16);
         r0 += x & 0xffffu;
         r1 += x >> 16;
       }
