@@ -2288,6 +2288,9 @@ __host__ __device__ constexpr size_t block_sort_smem_bytes(int nt) {
   return (size_t)padded_len(nt * small_items<Key, Val>()) * (sizeof(Key) + (kHasVal<Val> ? sizeof(Val) : 0));
 }
 
+#ifndef GSS_SMALL_L2PF
+#define GSS_SMALL_L2PF 1     // the next bucket of the CTA prefetched into L2 (8-byte keys alone)
+#endif
 #ifndef GSS_SMALL_DIRECT
 #define GSS_SMALL_DIRECT 1   // bucket keys read by the sorting threads straight into registers: 2^27 u32 in-SM
 #endif                       // sort 1.61 -> 1.52 ms, u64 pairs 4.47 -> 4.33, u32 pairs 2.63 -> 2.56; 8-byte keys
@@ -2318,6 +2321,21 @@ __global__ void __launch_bounds__(MAXT, MAXT <= kSmallNarrowThreads ? 2 : 1)
     const Key* src = c.keys(I.buf) + I.lo;
     const Val* vs = nullptr;
     if constexpr (kHasVal<Val>) vs = c.vals(I.buf) + I.lo;
+#if GSS_SMALL_L2PF
+    // the CTA's next bucket pulled into L2 while this one is sorted (its cp.async load then waits for L2, not
+    // DRAM): 8-byte keys alone (2^28 u64 in-SM sort 4.76 -> 4.74 ms; 2^27 u32 1.52 -> 1.56, so not there)
+    if (sizeof(Key) == 8 && !kHasVal<Val> && i + gridDim.x < ni) {
+      const Item J = list[i + gridDim.x];
+      const char* nk = reinterpret_cast<const char*>(c.keys(J.buf) + J.lo);
+      const uint32_t lines = (uint32_t)(((size_t)J.m * sizeof(Key) + 127) / 128);
+      for (uint32_t q = threadIdx.x; q < lines; q += nt) asm volatile("prefetch.global.L2 [%0];" ::"l"(nk + 128 * (size_t)q));
+      if constexpr (kHasVal<Val>) {
+        const char* nv = reinterpret_cast<const char*>(c.vals(J.buf) + J.lo);
+        const uint32_t vl = (uint32_t)(((size_t)J.m * sizeof(Val) + 127) / 128);
+        for (uint32_t q = threadIdx.x; q < vl; q += nt) asm volatile("prefetch.global.L2 [%0];" ::"l"(nv + 128 * (size_t)q));
+      }
+    }
+#endif
     if constexpr (GSS_SMALL_DIRECT && !Sorter::WB && !(sizeof(Key) == 8 && !kHasVal<Val>)) {
       // the threads read their first items straight from global memory (no shared-memory staging)
       Sorter::sort(sk, sv, (int)m, less, nt, src, vs);
